@@ -1,0 +1,333 @@
+#!/usr/bin/env python
+"""LM-OSEM subset-iteration benchmark (BASELINE.json metric: events/s per subset at the
+paper's 150x150x280 shape; s/recon).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl lmosem|reference] [--config C2]
+
+A step is one subset iteration (fused projection, c all-reduce when N > 1, update) of
+one 10^6-event subset; steps cycle through the config's 10 subsets. Inputs (events,
+norm, f) are resident in HBM before the timed region. L2 is flushed (a 256 MB write)
+before every timed step, outside the step's CUDA events. Rank 0 prints ONE JSON line.
+N > 1 is launched by torchrun (one process per GPU, NCCL).
+
+--impl reference times the float64 CPU oracle (the only reference this paper-only
+workload has) on rank 0, each step a bounded sample of the same subset.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import lmgen  # noqa: E402
+
+METRIC = "LM-OSEM events/s per subset (150x150x280)"
+# mean exact-Siddon path length per event (voxels) for the generated inputs
+# (tools/path_stats.py, oracle on a 20k-event sample)
+MEAN_PATH = {"C1": 25.37, "C2": 252.19, "C3": 252.19, "C4": 506.79, "C5": 440.96}
+FLUSH_BYTES = 256 << 20
+
+
+def env_int(k, d):
+    return int(os.environ.get(k, d))
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--impl", default="lmosem", choices=["lmosem", "reference"])
+    ap.add_argument("--config", default=None, help="C2 (N=1 default), C3 (N>1 default), C4, C5")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--cpu-sample", type=int, default=200_000, help="events in the oracle's timed sample")
+    return ap.parse_args()
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled every 200 ms during the timed region."""
+
+    Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+         "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.proc = None
+        self.lines = []
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.Q}",
+                                          "--format=csv,noheader,nounits", "-lms", "200"],
+                                         stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except OSError:
+            self.proc = None
+        return self
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def __exit__(self, *a):
+        if self.proc is not None:
+            time.sleep(0.25)
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except subprocess.TimeoutExpired:
+                self.proc.kill()
+
+    def summary(self):
+        sm, mx, reasons = [], 0.0, set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for ln in self.lines:
+            p = [x.strip() for x in ln.split(",")]
+            if len(p) < 6:
+                continue
+            try:
+                sm.append(float(p[0]))
+                mx = max(mx, float(p[1]))
+            except ValueError:
+                continue
+            for n, v in zip(names, p[2:6]):
+                if v.lower() == "active":
+                    reasons.add(n)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": mx or None,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+def measured_peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as fh:
+            return json.load(fh), "measured"
+    except OSError:
+        return {"hbm_gbs": 6650.0}, "fallback"
+
+
+def l2_peak_gbs(V: int):
+    """Live microbenchmark of random fp32 gather+RED pairs on a V-float buffer (the
+    projection's L2 access mix); returns (pair ops/s, GB/s at 8 B per pair)."""
+    import ctypes
+    from paper_conf_ipps_steuwerkg12_b200 import build as b
+    lib = ctypes.CDLL(b.L2PEAK_SO)
+    lib.l2peak_run.argtypes = [ctypes.c_int, ctypes.c_int64, ctypes.c_int32, ctypes.POINTER(ctypes.c_float),
+                               ctypes.POINTER(ctypes.c_double)]
+    out = {}
+    for name, mode in (("red", 0), ("ldg", 1), ("pair", 2), ("pair_run8", 4)):
+        ms, ops = ctypes.c_float(), ctypes.c_double()
+        if lib.l2peak_run(mode, V, 256, ctypes.byref(ms), ctypes.byref(ops)) != 0:
+            return None
+        out[name] = ops.value / (ms.value * 1e-3)
+    return out
+
+
+def cpu_baseline(cfg, sample: int):
+    """The float64 oracle as it stands, on this host's cores, on a bounded sample."""
+    import oracle
+    ev = lmgen.subset_events(cfg, 0, sample)
+    s = lmgen.norm(cfg)
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    f0 = np.ones(cfg.n_voxels)
+    t0 = time.perf_counter()
+    oracle.subset_step(g, ev, s, f0)
+    dt = time.perf_counter() - t0
+    return {"value": sample / dt, "unit": "events/s", "cores": oracle.get_threads(), "kind": "oracle",
+            "sample": f"{sample} events of subset 0 of {cfg.name} (one subset step incl. the {cfg.n_voxels}-voxel "
+                      f"update), {dt:.2f} s wall"}
+
+
+def run_reference(args, cfg, rank):
+    if rank != 0:
+        return
+    import oracle
+    sample = min(args.cpu_sample, cfg.n_events)
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    s = lmgen.norm(cfg)
+    evs = [lmgen.subset_events(cfg, l % cfg.n_subsets, sample) for l in range(min(cfg.n_subsets, args.warmup + args.steps))]
+    f = np.ones(cfg.n_voxels)
+    for k in range(args.warmup):
+        f = oracle.subset_step(g, evs[k % len(evs)], s, f)
+    t0 = time.perf_counter()
+    for k in range(args.steps):
+        f = oracle.subset_step(g, evs[(args.warmup + k) % len(evs)], s, f)
+    dt = time.perf_counter() - t0
+    v = sample * args.steps / dt
+    cores = oracle.get_threads()
+    line = {"metric": METRIC, "value": v, "unit": "events/s", "impl": "reference", "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * dt / args.steps,
+            "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
+            "data": "synthetic", "config": {"workload": f"{cfg.name}: {cfg.note} {cfg.dims[0]}x{cfg.dims[1]}x"
+                                            f"{cfg.dims[2]}, subsets of {cfg.n_events} events (oracle steps use a "
+                                            f"{sample}-event sample of each subset)"},
+            "cpu_baseline": {"value": v, "unit": "events/s", "cores": cores, "kind": "oracle",
+                             "sample": f"{sample} events per step x {args.steps} steps"},
+            "e2e": {"value": v, "unit": "events/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def main():
+    args = parse()
+    world = env_int("WORLD_SIZE", 1)
+    rank = env_int("RANK", 0)
+    local = env_int("LOCAL_RANK", 0)
+    name = args.config or ("C2" if world == 1 else "C3")
+    cfg = lmgen.CONFIGS[name]
+    if args.impl == "reference":
+        return run_reference(args, cfg, rank)
+
+    import torch
+    import torch.distributed as dist
+
+    import paper_conf_ipps_steuwerkg12_b200 as pkg
+
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    dev = torch.device("cuda", local)
+
+    # ---- inputs, resident in HBM (every rank holds the whole subsets; the library
+    # projects its block: PAPER.md lines 503-505, block distribution)
+    L = cfg.n_subsets
+    ev_host = lmgen.events(cfg, 0, cfg.n_events * L)
+    s_host = lmgen.norm(cfg)
+    ev = torch.from_numpy(ev_host).to(dev)
+    norm = torch.from_numpy(s_host).to(dev)
+    f = torch.ones(cfg.n_voxels, device=dev)
+    flush = torch.empty(FLUSH_BYTES // 4, device=dev)
+    stream = torch.cuda.current_stream()
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, norm, dist=pkg.make_dist(rank, world), stream=stream)
+    N = cfg.n_events
+
+    def subset(k):
+        l = k % L
+        return ev[l * N:(l + 1) * N]
+
+    for k in range(args.warmup):
+        rec.subset_step(subset(k), f)
+    rec.synchronize()
+
+    starts = [torch.cuda.Event(enable_timing=True) for _ in range(args.steps)]
+    ends = [torch.cuda.Event(enable_timing=True) for _ in range(args.steps)]
+    launches0 = rec.stats()["launches"]
+    rec.set_timing(True)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    with ClockSampler(local) as clk:
+        t_wall = time.perf_counter()
+        for k in range(args.steps):
+            flush.fill_(float(k))                # L2 flush, outside the step's events
+            starts[k].record(stream)
+            rec.subset_step(subset(args.warmup + k), f)
+            ends[k].record(stream)
+        torch.cuda.synchronize()
+        if world > 1:
+            dist.barrier()
+        t_wall = time.perf_counter() - t_wall
+    st = rec.stats()
+    rec.set_timing(False)
+    step_ms = [a.elapsed_time(b) for a, b in zip(starts, ends)]
+    tot_ms = sum(step_ms)
+    t = torch.tensor([tot_ms, st["project_ms"], st["combine_ms"], st["update_ms"]], device=dev, dtype=torch.float64)
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    tot_ms, proj_ms, comb_ms, upd_ms = (float(x) for x in t.tolist())
+    K = args.steps
+    value = N * K / (tot_ms * 1e-3)  # events of the whole job (each subset's N split over ranks)
+
+    # ---- e2e through the public API with HOST buffers: one host reconstruction over the
+    # K subsets (pinned events streamed per subset, f uploaded and downloaded)
+    e2e = None
+    if not args.no_e2e:
+        pinned = torch.from_numpy(ev_host).pin_memory()
+        offs = np.arange(L + 1, dtype=np.int64) * N
+        fh = np.ones(cfg.n_voxels, np.float32)
+        rec.reconstruct_host(pinned, offs[:2], 1, fh)  # warm-up (allocates the streaming buffers)
+        reps = max(1, K // L)
+        if world > 1:
+            dist.barrier()
+        t0 = time.perf_counter()
+        for _ in range(reps):
+            rec.reconstruct_host(pinned, offs, 1, fh)
+        te = torch.tensor([time.perf_counter() - t0], dtype=torch.float64, device=dev)
+        if world > 1:
+            dist.all_reduce(te, op=dist.ReduceOp.MAX)
+        b, e = pkg.block_range(N, rank, world)
+        e2e = {"value": N * L * reps / float(te.item()), "unit": "events/s",
+               "h2d_bytes_per_step": int(24 * (e - b) + 4 * cfg.n_voxels / L),
+               "d2h_bytes_per_step": int(4 * cfg.n_voxels / L),
+               "note": f"lmosem_reconstruct_host over {L} subsets x {reps} (pinned host events streamed per subset, "
+                       f"overlapped with projection; f H2D/D2H once per reconstruction), wall clock"}
+        s_recon = float(te.item()) / reps
+    else:
+        s_recon = None
+
+    if rank != 0:
+        rec.close()
+        if world > 1:
+            dist.destroy_process_group()
+        return
+
+    peaks, peak_kind = measured_peaks()
+    mean_path = MEAN_PATH[name]
+    ev_per_launch = N / world
+    pairs = ev_per_launch * mean_path
+    proj_avg_s = proj_ms / K * 1e-3
+    l2 = l2_peak_gbs(cfg.n_voxels)
+    alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0  # 4 B gather + 4 B RED per path element, 24 B/event
+    roof = {"kernel": "k_project<0> (fused Siddon + forward + back-projection)", "bound": "l2",
+            "achieved": alg_l2_bytes / proj_avg_s / 1e9, "unit": "GB/s", "traffic": None,
+            "per_unit": f"{mean_path} path elements x (4 B f gather + 4 B c RED) + 24 B event per event",
+            "units_per_launch": ev_per_launch}
+    if l2:
+        roof["peak"] = l2["pair"] * 8.0 / 1e9
+        roof["peak_kind"] = ("measured live: random fp32 gather+RED pairs on a V-float L2-resident buffer "
+                             "(libl2peak.so, PAIR_RANDOM)")
+        roof["frac"] = roof["achieved"] / roof["peak"]
+        roof["l2_micro_ops_per_s"] = l2
+    hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0) / proj_avg_s / 1e9, "peak": peaks["hbm_gbs"],
+           "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
+    hbm["frac"] = hbm["achieved"] / hbm["peak"]
+    upd_bytes = 20.0 * cfg.n_voxels  # read f, c, s; write f, c
+    upd = {"bound": "hbm", "achieved": upd_bytes / (upd_ms / K * 1e-3) / 1e9, "peak": peaks["hbm_gbs"],
+           "unit": "GB/s", "peak_kind": peak_kind, "what": "k_update (20 B/voxel)"}
+    upd["frac"] = upd["achieved"] / upd["peak"]
+
+    line = {
+        "metric": METRIC, "value": value, "unit": "events/s", "n_gpus": world, "steps": K, "warmup": args.warmup,
+        "ms_per_step": tot_ms / K, "higher_is_better": True, "scaling": "strong", "vs_baseline": None,
+        "dtype": "f32", "geometry_dtype": "f64", "data": "synthetic",
+        "config": {"workload": f"{name}: {cfg.note} LM-OSEM {cfg.dims[0]}x{cfg.dims[1]}x{cfg.dims[2]} @ "
+                               f"{cfg.voxel_mm[0]} mm, {L} subsets x {N} events, 1 iteration",
+                   "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block, f copy, c allreduce)",
+                   "l2": "flushed before every timed step (256 MB write outside the step events)"},
+        "s_per_recon": tot_ms / K * L * 1e-3, "s_per_recon_e2e": s_recon,
+        "phase_ms_per_step": {"project": proj_ms / K, "combine": comb_ms / K, "update": upd_ms / K},
+        "roofline": roof, "roofline_hbm_events": hbm, "roofline_update": upd,
+        "gpu_launches": int(st["launches"] - launches0),
+        "clocks": clk.summary(), "wall_s_timed_region": t_wall,
+        "e2e": e2e,
+    }
+    if not args.no_cpu_baseline and world == 1:
+        line["cpu_baseline"] = cpu_baseline(cfg, min(args.cpu_sample, N))
+    print(json.dumps(line), flush=True)
+    rec.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

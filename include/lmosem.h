@@ -1,0 +1,163 @@
+/* lmosem.h — C ABI of the B200-native LM-OSEM subset iteration.
+ *
+ * The operation (§IV, Listing 2; Listing 3):
+ * list-mode OSEM reconstructs an image f from events (lines of response, LORs) split
+ * into subsets. One subset iteration is
+ *   step 1 (Listing 2 lines 5-13): c <- 0; for every event i of the subset,
+ *            path_i = compute_path(event_i)                   exact Siddon chord lengths a_ij
+ *            fp_i   = sum_j a_ij f_j                          forward projection
+ *            c_j   += a_ij / fp_i  for j on path_i            back-projection (skip fp_i <= 0)
+ *   combine (Listing 3 lines 6, 15-16): with several GPUs the
+ *            per-GPU error images are added element-wise (copy(add) distribution)
+ *   step 2 (Listing 2 lines 16-17 with the norm of BASELINE.json north_star):
+ *            f_j <- f_j * c_j / s_j  where c_j > 0 and s_j > 0, else unchanged.
+ * Readings of points the paper leaves open are listed in DESIGN.md (S1-S17).
+ *
+ * Conventions
+ *  - Volume: nx*ny*nz voxels of vx*vy*vz mm, centred on the origin. Voxel (ix,iy,iz) is
+ *    the half-open box [x0+ix*vx, x0+(ix+1)*vx) x ..., x0 = -nx*vx/2; images are float32
+ *    with linear index j = ix + nx*(iy + ny*iz) (x fastest). V = nx*ny*nz < 2^31.
+ *  - Event: lmosem_event, 6 float32 (two detection points in mm, the segment p1 -> p2).
+ *    Non-finite, zero-length or volume-missing events, and events with fp_i <= 0,
+ *    contribute nothing (not an error).
+ *  - Pointers: "device" = CUDA device memory of the context's device; "host" = host
+ *    memory (pinned memory gives overlapped copies). The caller owns every buffer it
+ *    passes; the context owns c, its copy of the norm image, scratch buffers, its
+ *    streams and (world > 1) its NCCL communicator.
+ *  - Ordering: calls taking device buffers are enqueued on the context's stream (see
+ *    lmosem_set_stream) and return without waiting; lmosem_synchronize waits. Calls
+ *    taking host buffers are synchronous.
+ *  - Distribution (§III.A; §IV.A): with
+ *    world > 1, subset_step / reconstruct are collective. Every rank passes the WHOLE
+ *    subset; rank r projects the block [floor(r*N/P), floor((r+1)*N/P)) (block
+ *    distribution), f is replicated (copy distribution) and c is combined by an NCCL
+ *    all-reduce(sum) (copy(add)). Every rank then applies step 2 to its full replica,
+ *    so the replicas stay identical.
+ *  - Errors: every call returns a status. EINVAL for bad arguments (nothing enqueued);
+ *    ECUDA/ENCCL for runtime failures (message in lmosem_last_error), after which the
+ *    context answers ESTATE to everything except lmosem_last_error and lmosem_destroy.
+ *  - Threading: one host thread per context; one context per GPU (rank).
+ */
+#ifndef LMOSEM_H
+#define LMOSEM_H
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct lmosem_ctx lmosem_ctx;
+
+/* One list-mode event: a line of response between two detection points (mm). */
+typedef struct {
+    float x1, y1, z1, x2, y2, z2;
+} lmosem_event;
+
+typedef enum {
+    LMOSEM_OK = 0,
+    LMOSEM_EINVAL = 1,
+    LMOSEM_ENOMEM = 2,
+    LMOSEM_ECUDA = 3,
+    LMOSEM_ENCCL = 4,
+    LMOSEM_ESTATE = 5
+} lmosem_status;
+
+#define LMOSEM_NCCL_ID_BYTES 128
+
+/* Multi-GPU setup; pass NULL (or world == 1) for a single GPU. nccl_unique_id points to
+ * LMOSEM_NCCL_ID_BYTES bytes produced by lmosem_nccl_unique_id on one rank and broadcast
+ * to all (the Python binding uses torch.distributed for the broadcast). */
+typedef struct {
+    int32_t rank, world;
+    const void* nccl_unique_id;
+} lmosem_dist;
+
+/* Per-context counters. Phase times are summed CUDA-event durations (ms) on the
+ * context's stream, recorded only while timing is enabled (lmosem_set_timing). */
+typedef struct {
+    int64_t launches;      /* kernels this context launched (all time) */
+    int64_t subsets;       /* subset iterations completed (all time) */
+    int64_t events;        /* events projected by this rank (all time) */
+    int64_t timed_subsets; /* subsets covered by the phase times below */
+    double project_ms;     /* step 1: fused traversal + forward + back-projection kernel */
+    double combine_ms;     /* c all-reduce (world > 1) */
+    double update_ms;      /* step 2: update kernel (also re-zeroes c) */
+    double h2d_ms;         /* event uploads in lmosem_reconstruct_host (copy stream) */
+} lmosem_stats;
+
+/* Library version as "lmosem <major>.<minor> sm_100a". */
+const char* lmosem_version(void);
+
+/* Block distribution: the event range [begin, end) of rank r of
+ * world P for n events: begin = floor(r*n/P), end = floor((r+1)*n/P). Host only, no GPU
+ * needed. EINVAL if n < 0, world < 1, rank outside [0, world) or a pointer is NULL. */
+lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end);
+
+/* Writes a fresh NCCL unique id (LMOSEM_NCCL_ID_BYTES bytes) to out. ENCCL on failure. */
+lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
+
+/* Creates a context on the current CUDA device.
+ *   dims[3]     = {nx, ny, nz} > 0, V < 2^31
+ *   voxel_mm[3] = voxel size in mm, finite and > 0
+ *   norm        = V float32 sensitivity image s (device or host); copied, caller keeps it
+ *   dist        = NULL for one GPU, else the rank/world/NCCL id (collective init)
+ * Returns EINVAL / ENOMEM / ECUDA / ENCCL; *out is NULL on failure. */
+lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
+                          const float* norm, const lmosem_dist* dist);
+
+/* Uses the given cudaStream_t (as void*) for all later device work; NULL restores the
+ * context's own stream. The stream must belong to the context's device. */
+lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream);
+
+/* One subset iteration (step 1, combine, step 2) over n_events device events; f is the
+ * V float32 device image, updated in place. Stream-ordered. n_events == 0 leaves f
+ * unchanged (c stays 0). */
+lmosem_status lmosem_subset_step(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events, float* f);
+
+/* n_iterations passes over subsets l = 0..n_subsets-1 in order; subset l is
+ * events[offsets[l], offsets[l+1]) (offsets: host, n_subsets+1 non-decreasing int64,
+ * offsets[0] >= 0). events and f are device buffers. Stream-ordered. */
+lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
+                                 int32_t n_subsets, int32_t n_iterations, float* f);
+
+/* As lmosem_reconstruct with HOST events and HOST f (in: f0, out: result). Uploads f,
+ * streams each subset's events (this rank's block only) to the device on a copy stream,
+ * double-buffered so the upload of subset l+1 overlaps the projection of subset l,
+ * downloads f. Synchronous. */
+lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
+                                      int32_t n_subsets, int32_t n_iterations, float* f);
+
+/* Step 1 only, for tests: c_out (V float32, device) <- error image of n_events device
+ * events against device image f (c starts from 0; no combine, no update). */
+lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
+                                 const float* f, float* c_out);
+
+/* Forward projection only, for tests: fp_out[i] = sum_j a_ij f_j (float32, device). */
+lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
+                             const float* f, float* fp_out);
+
+/* Step 2 only, for tests: f_j <- f_j*c_j/s_j where c_j > 0 and s_j > 0 (device f and c,
+ * the context's norm); c is re-zeroed. */
+lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c);
+
+/* Waits for all work enqueued by this context. Reports asynchronous kernel faults. */
+lmosem_status lmosem_synchronize(lmosem_ctx* ctx);
+
+/* Enables (1) / disables (0) per-phase CUDA-event timing; enabling clears the times. */
+lmosem_status lmosem_set_timing(lmosem_ctx* ctx, int32_t enable);
+
+/* Resolves pending timing events (synchronizes) and copies the counters to *out. */
+lmosem_status lmosem_get_stats(lmosem_ctx* ctx, lmosem_stats* out);
+
+/* Releases everything the context owns (synchronizes first). NULL is a no-op. */
+lmosem_status lmosem_destroy(lmosem_ctx* ctx);
+
+/* Last error message of ctx ("" if none). With ctx == NULL: the message of the last
+ * failed lmosem_init on the calling thread. */
+const char* lmosem_last_error(const lmosem_ctx* ctx);
+
+#ifdef __cplusplus
+}
+#endif
+#endif

@@ -1,0 +1,92 @@
+// l2peak.cu — microbenchmarks for the L2 roofline denominators (include/l2peak.h).
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "l2peak.h"
+
+#define L2PEAK_API extern "C" __attribute__((visibility("default")))
+
+namespace {
+
+__device__ __forceinline__ uint32_t hash32(uint32_t x) {
+    x ^= x >> 16; x *= 0x7feb352dU; x ^= x >> 15; x *= 0x846ca68bU; x ^= x >> 16;
+    return x;
+}
+
+template <int MODE>
+__global__ void __launch_bounds__(256) k_l2(float* __restrict__ buf, const float* __restrict__ src, uint32_t n,
+                                            int ops, float* __restrict__ sink) {
+    const uint32_t tid = blockIdx.x * blockDim.x + threadIdx.x;
+    const int lane = threadIdx.x & 31;
+    float acc = 0.f;
+#pragma unroll 4
+    for (int it = 0; it < ops; ++it) {
+        uint32_t h = hash32(tid * 0x9E3779B9u + (uint32_t)it * 0x85EBCA6Bu);
+        uint32_t j;
+        if (MODE == L2PEAK_RED_RUN8 || MODE == L2PEAK_PAIR_RUN8) {
+            uint32_t g = hash32((tid >> 3) * 0x9E3779B9u + (uint32_t)it * 0x85EBCA6Bu);
+            j = (uint32_t)(((uint64_t)g * (n - 8)) >> 32) + (lane & 7);
+        } else {
+            j = (uint32_t)(((uint64_t)h * n) >> 32);
+        }
+        if (MODE == L2PEAK_LDG_RANDOM || MODE == L2PEAK_PAIR_RANDOM || MODE == L2PEAK_PAIR_RUN8)
+            acc += __ldg(src + j);
+        if (MODE != L2PEAK_LDG_RANDOM) atomicAdd(buf + j, 1.0f + acc * 0.0f);
+    }
+    if (acc == 12345.678f) sink[0] = acc;  // keeps the gathers alive
+}
+
+template <int MODE>
+cudaError_t launch(float* buf, const float* src, uint32_t n, int ops, float* sink, int grid) {
+    k_l2<MODE><<<grid, 256>>>(buf, src, n, ops, sink);
+    return cudaGetLastError();
+}
+
+cudaError_t launch_mode(int mode, float* buf, const float* src, uint32_t n, int ops, float* sink, int grid) {
+    switch (mode) {
+        case L2PEAK_RED_RANDOM: return launch<L2PEAK_RED_RANDOM>(buf, src, n, ops, sink, grid);
+        case L2PEAK_LDG_RANDOM: return launch<L2PEAK_LDG_RANDOM>(buf, src, n, ops, sink, grid);
+        case L2PEAK_PAIR_RANDOM: return launch<L2PEAK_PAIR_RANDOM>(buf, src, n, ops, sink, grid);
+        case L2PEAK_RED_RUN8: return launch<L2PEAK_RED_RUN8>(buf, src, n, ops, sink, grid);
+        case L2PEAK_PAIR_RUN8: return launch<L2PEAK_PAIR_RUN8>(buf, src, n, ops, sink, grid);
+    }
+    return cudaErrorInvalidValue;
+}
+
+}  // namespace
+
+L2PEAK_API int l2peak_run(int mode, int64_t n_floats, int32_t ops_per_thread, float* ms, double* ops) {
+    if (mode < 0 || mode > 4 || n_floats < 64 || n_floats >= (int64_t(1) << 32) || ops_per_thread <= 0 || !ms || !ops)
+        return -1;
+    int dev = 0, sms = 0, per_sm = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess) return -1;
+    if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess) return -1;
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_l2<L2PEAK_PAIR_RANDOM>, 256, 0);
+    if (per_sm < 1) per_sm = 1;
+    const int grid = sms * per_sm;
+    float *buf = nullptr, *src = nullptr, *sink = nullptr;
+    cudaEvent_t e0 = nullptr, e1 = nullptr;
+    int rc = -1;
+    if (cudaMalloc(&buf, sizeof(float) * n_floats) != cudaSuccess) goto done;
+    if (cudaMalloc(&src, sizeof(float) * n_floats) != cudaSuccess) goto done;
+    if (cudaMalloc(&sink, sizeof(float)) != cudaSuccess) goto done;
+    cudaMemset(buf, 0, sizeof(float) * n_floats);
+    cudaMemset(src, 0, sizeof(float) * n_floats);
+    cudaEventCreate(&e0);
+    cudaEventCreate(&e1);
+    if (launch_mode(mode, buf, src, (uint32_t)n_floats, ops_per_thread, sink, grid) != cudaSuccess) goto done;
+    cudaEventRecord(e0);
+    if (launch_mode(mode, buf, src, (uint32_t)n_floats, ops_per_thread, sink, grid) != cudaSuccess) goto done;
+    cudaEventRecord(e1);
+    if (cudaEventSynchronize(e1) != cudaSuccess) goto done;
+    cudaEventElapsedTime(ms, e0, e1);
+    *ops = (double)grid * 256.0 * ops_per_thread;
+    rc = 0;
+done:
+    if (e0) cudaEventDestroy(e0);
+    if (e1) cudaEventDestroy(e1);
+    cudaFree(buf);
+    cudaFree(src);
+    cudaFree(sink);
+    return rc;
+}

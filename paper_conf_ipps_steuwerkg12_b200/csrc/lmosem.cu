@@ -1,0 +1,465 @@
+// lmosem.cu — context, C ABI (include/lmosem.h) and launch logic of the B200-native
+// LM-OSEM subset iteration (§IV, Listings 2-3). Kernels: lmosem_kernels.cuh.
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstdio>
+#include <cstring>
+#include <new>
+#include <string>
+#include <vector>
+
+#include "lmosem.h"
+#include "lmosem_kernels.cuh"
+
+#define LMOSEM_API extern "C" __attribute__((visibility("default")))
+
+namespace {
+
+thread_local std::string g_init_err;  // message of the last failed lmosem_init on this thread
+
+struct PhaseMarks {
+    cudaEvent_t e[4];  // start, after project, after combine, after update
+};
+
+}  // namespace
+
+struct lmosem_ctx {
+    int device = -1;
+    int32_t dims[3] = {0, 0, 0};
+    float vox[3] = {0, 0, 0};
+    int64_t V = 0;
+    lmk::GridGeom geom{};
+    float* c = nullptr;     // error image (kept all-zero between subsets)
+    float* norm = nullptr;  // copy of s
+    cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
+    int rank = 0, world = 1;
+    ncclComm_t comm = nullptr;
+    int num_sms = 0, proj_blocks_per_sm = 0, upd_blocks = 0;
+    bool failed = false;
+    std::string err;
+    // timing
+    bool timing = false;
+    std::vector<PhaseMarks> pending, pool;
+    std::vector<cudaEvent_t> h2d_pending, h2d_pool;
+    lmosem_stats st{};
+    // host-streaming resources
+    lmosem_event* dev_ev[2] = {nullptr, nullptr};
+    int64_t dev_ev_cap = 0;
+    float* dev_f = nullptr;
+    cudaEvent_t ev_copied[2] = {nullptr, nullptr}, ev_consumed[2] = {nullptr, nullptr};
+};
+
+namespace {
+
+lmosem_status fail(lmosem_ctx* ctx, lmosem_status s, const std::string& msg) {
+    if (ctx) {
+        ctx->err = msg;
+        if (s == LMOSEM_ECUDA || s == LMOSEM_ENCCL) ctx->failed = true;
+    }
+    return s;
+}
+
+#define CK(call)                                                                                    \
+    do {                                                                                            \
+        cudaError_t e_ = (call);                                                                    \
+        if (e_ != cudaSuccess)                                                                      \
+            return fail(ctx, LMOSEM_ECUDA, std::string(#call) + ": " + cudaGetErrorString(e_));     \
+    } while (0)
+
+#define NK(call)                                                                                    \
+    do {                                                                                            \
+        ncclResult_t r_ = (call);                                                                   \
+        if (r_ != ncclSuccess)                                                                      \
+            return fail(ctx, LMOSEM_ENCCL, std::string(#call) + ": " + ncclGetErrorString(r_));     \
+    } while (0)
+
+#define USABLE(ctx)                                                                                 \
+    do {                                                                                            \
+        if (!(ctx)) return LMOSEM_EINVAL;                                                           \
+        if ((ctx)->failed) return LMOSEM_ESTATE;                                                    \
+    } while (0)
+
+void block_range(int64_t n, int r, int P, int64_t* b, int64_t* e) {
+    // floor(r*n/P) without overflow for n < 2^62 / P
+    *b = (int64_t)((__int128)n * r / P);
+    *e = (int64_t)((__int128)n * (r + 1) / P);
+}
+
+lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, const float* f, float* c,
+                             float* fp_out, int mode) {
+    if (n <= 0) return LMOSEM_OK;
+    const int64_t warps_needed = (n + 31) / 32;
+    const int64_t blocks_needed = (warps_needed + 7) / 8;
+    const int64_t cap = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm;
+    const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
+    const float* evf = reinterpret_cast<const float*>(ev);
+    if (mode == 0)
+        lmk::k_project<0><<<grid, 256, 0, ctx->stream>>>(evf, n, f, c, nullptr, ctx->geom);
+    else
+        lmk::k_project<1><<<grid, 256, 0, ctx->stream>>>(evf, n, f, nullptr, fp_out, ctx->geom);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return LMOSEM_OK;
+}
+
+lmosem_status launch_update(lmosem_ctx* ctx, float* f, float* c) {
+    const int vec = ((((uintptr_t)f) | ((uintptr_t)c) | ((uintptr_t)ctx->norm)) & 15) == 0;
+    lmk::k_update<<<ctx->upd_blocks, 256, 0, ctx->stream>>>(f, c, ctx->norm, ctx->V, vec);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return LMOSEM_OK;
+}
+
+lmosem_status mark(lmosem_ctx* ctx, PhaseMarks* pm, int k) {
+    if (pm) CK(cudaEventRecord(pm->e[k], ctx->stream));
+    return LMOSEM_OK;
+}
+
+lmosem_status get_marks(lmosem_ctx* ctx, PhaseMarks** out) {
+    *out = nullptr;
+    if (!ctx->timing) return LMOSEM_OK;
+    if (ctx->pool.empty()) {
+        PhaseMarks pm;
+        for (int k = 0; k < 4; ++k) CK(cudaEventCreate(&pm.e[k]));
+        ctx->pool.push_back(pm);
+    }
+    ctx->pending.push_back(ctx->pool.back());
+    ctx->pool.pop_back();
+    *out = &ctx->pending.back();
+    return LMOSEM_OK;
+}
+
+// One subset iteration on the context's stream: this rank's block of step 1, the c
+// all-reduce (copy(add) -> every rank has the sum), step 2 on the full replica.
+lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* f, bool whole_subset) {
+    int64_t b = 0, e = n;
+    if (whole_subset) block_range(n, ctx->rank, ctx->world, &b, &e);
+    PhaseMarks* pm = nullptr;
+    lmosem_status s;
+    if ((s = get_marks(ctx, &pm))) return s;
+    if ((s = mark(ctx, pm, 0))) return s;
+    if ((s = launch_project(ctx, ev + b, e - b, f, ctx->c, nullptr, 0))) return s;
+    if ((s = mark(ctx, pm, 1))) return s;
+    if (ctx->world > 1) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->V, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    if ((s = mark(ctx, pm, 2))) return s;
+    if ((s = launch_update(ctx, f, ctx->c))) return s;
+    if ((s = mark(ctx, pm, 3))) return s;
+    ctx->st.subsets++;
+    ctx->st.events += e - b;
+    return LMOSEM_OK;
+}
+
+lmosem_status check_offsets(const int64_t* off, int32_t L) {
+    if (!off || L < 0) return LMOSEM_EINVAL;
+    if (off[0] < 0) return LMOSEM_EINVAL;
+    for (int32_t l = 0; l < L; ++l)
+        if (off[l + 1] < off[l]) return LMOSEM_EINVAL;
+    return LMOSEM_OK;
+}
+
+lmosem_status resolve_timing(lmosem_ctx* ctx) {
+    for (auto& pm : ctx->pending) {
+        CK(cudaEventSynchronize(pm.e[3]));
+        float t01, t12, t23;
+        CK(cudaEventElapsedTime(&t01, pm.e[0], pm.e[1]));
+        CK(cudaEventElapsedTime(&t12, pm.e[1], pm.e[2]));
+        CK(cudaEventElapsedTime(&t23, pm.e[2], pm.e[3]));
+        ctx->st.project_ms += t01;
+        ctx->st.combine_ms += t12;
+        ctx->st.update_ms += t23;
+        ctx->st.timed_subsets++;
+        ctx->pool.push_back(pm);
+    }
+    ctx->pending.clear();
+    for (size_t k = 0; k + 1 < ctx->h2d_pending.size(); k += 2) {
+        CK(cudaEventSynchronize(ctx->h2d_pending[k + 1]));
+        float t;
+        CK(cudaEventElapsedTime(&t, ctx->h2d_pending[k], ctx->h2d_pending[k + 1]));
+        ctx->st.h2d_ms += t;
+        ctx->h2d_pool.push_back(ctx->h2d_pending[k]);
+        ctx->h2d_pool.push_back(ctx->h2d_pending[k + 1]);
+    }
+    ctx->h2d_pending.clear();
+    return LMOSEM_OK;
+}
+
+}  // namespace
+
+LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.1 sm_100a"; }
+
+LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end) {
+    if (!begin || !end || n < 0 || world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
+    block_range(n, rank, world, begin, end);
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_nccl_unique_id(void* out, size_t size) {
+    if (!out || size < sizeof(ncclUniqueId) || sizeof(ncclUniqueId) != LMOSEM_NCCL_ID_BYTES) return LMOSEM_EINVAL;
+    ncclUniqueId id;
+    if (ncclGetUniqueId(&id) != ncclSuccess) return LMOSEM_ENCCL;
+    std::memcpy(out, &id, sizeof(id));
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
+                                     const float* norm, const lmosem_dist* dist) {
+    if (!out) return LMOSEM_EINVAL;
+    *out = nullptr;
+    if (!dims || !voxel_mm || !norm) return LMOSEM_EINVAL;
+    int64_t V = 1;
+    for (int k = 0; k < 3; ++k) {
+        if (dims[k] <= 0) return LMOSEM_EINVAL;
+        if (!std::isfinite(voxel_mm[k]) || !(voxel_mm[k] > 0.0f)) return LMOSEM_EINVAL;
+        V *= dims[k];
+    }
+    if (V >= (int64_t(1) << 31)) return LMOSEM_EINVAL;
+    int rank = 0, world = 1;
+    if (dist) {
+        rank = dist->rank;
+        world = dist->world;
+        if (world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
+        if (world > 1 && !dist->nccl_unique_id) return LMOSEM_EINVAL;
+    }
+    lmosem_ctx* ctx = new (std::nothrow) lmosem_ctx;
+    if (!ctx) return LMOSEM_ENOMEM;
+    auto bail = [&](lmosem_status s) {
+        g_init_err = ctx->err;
+        lmosem_destroy(ctx);
+        return s;
+    };
+    ctx->V = V;
+    ctx->rank = rank;
+    ctx->world = world;
+    for (int k = 0; k < 3; ++k) {
+        ctx->dims[k] = dims[k];
+        ctx->vox[k] = voxel_mm[k];
+        ctx->geom.n[k] = dims[k];
+        ctx->geom.lo[k] = -0.5 * (double)dims[k] * (double)voxel_mm[k];
+        ctx->geom.inv_v[k] = 1.0 / (double)voxel_mm[k];
+    }
+    ctx->geom.stride[0] = 1;
+    ctx->geom.stride[1] = dims[0];
+    ctx->geom.stride[2] = dims[0] * dims[1];
+
+    lmosem_status s = LMOSEM_OK;
+    auto cuda = [&](cudaError_t e, const char* what) {
+        if (e != cudaSuccess && s == LMOSEM_OK) {
+            s = (e == cudaErrorMemoryAllocation) ? LMOSEM_ENOMEM : LMOSEM_ECUDA;
+            ctx->err = std::string(what) + ": " + cudaGetErrorString(e);
+        }
+        return e == cudaSuccess;
+    };
+    if (!cuda(cudaGetDevice(&ctx->device), "cudaGetDevice")) return bail(s);
+    cudaDeviceProp prop;
+    if (!cuda(cudaGetDeviceProperties(&prop, ctx->device), "cudaGetDeviceProperties")) return bail(s);
+    ctx->num_sms = prop.multiProcessorCount;
+    cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, 256, 0),
+         "occupancy");
+    if (ctx->proj_blocks_per_sm < 1) ctx->proj_blocks_per_sm = 1;
+    ctx->upd_blocks = ctx->num_sms * 8;
+    cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
+    cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
+    ctx->stream = ctx->own_stream;
+    cuda(cudaMalloc(&ctx->c, sizeof(float) * V), "cudaMalloc(c)");
+    cuda(cudaMalloc(&ctx->norm, sizeof(float) * V), "cudaMalloc(norm)");
+    for (int k = 0; k < 2; ++k) {
+        cuda(cudaEventCreateWithFlags(&ctx->ev_copied[k], cudaEventDisableTiming), "cudaEventCreate");
+        cuda(cudaEventCreateWithFlags(&ctx->ev_consumed[k], cudaEventDisableTiming), "cudaEventCreate");
+    }
+    if (s != LMOSEM_OK) return bail(s);
+    cuda(cudaMemcpyAsync(ctx->norm, norm, sizeof(float) * V, cudaMemcpyDefault, ctx->stream), "copy norm");
+    cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * V, ctx->stream), "memset c");
+    cuda(cudaStreamSynchronize(ctx->stream), "sync");
+    if (s != LMOSEM_OK) return bail(s);
+    if (world > 1) {
+        ncclUniqueId id;
+        std::memcpy(&id, dist->nccl_unique_id, sizeof(id));
+        ncclResult_t r = ncclCommInitRank(&ctx->comm, world, id, rank);
+        if (r != ncclSuccess) {
+            ctx->comm = nullptr;
+            ctx->err = std::string("ncclCommInitRank: ") + ncclGetErrorString(r);
+            return bail(LMOSEM_ENCCL);
+        }
+    }
+    *out = ctx;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream) {
+    USABLE(ctx);
+    ctx->stream = stream ? (cudaStream_t)stream : ctx->own_stream;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_subset_step(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events, float* f) {
+    USABLE(ctx);
+    if (!f || n_events < 0 || (n_events > 0 && !events)) return fail(ctx, LMOSEM_EINVAL, "subset_step: bad arguments");
+    return subset_iteration(ctx, events, n_events, f, true);
+}
+
+LMOSEM_API lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
+                                            int32_t n_subsets, int32_t n_iterations, float* f) {
+    USABLE(ctx);
+    if (!f || n_iterations < 0 || check_offsets(offsets, n_subsets) || (offsets[n_subsets] > offsets[0] && !events))
+        return fail(ctx, LMOSEM_EINVAL, "reconstruct: bad arguments");
+    for (int32_t it = 0; it < n_iterations; ++it)
+        for (int32_t l = 0; l < n_subsets; ++l) {
+            lmosem_status s = subset_iteration(ctx, events + offsets[l], offsets[l + 1] - offsets[l], f, true);
+            if (s) return s;
+        }
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
+                                                 int32_t n_subsets, int32_t n_iterations, float* f) {
+    USABLE(ctx);
+    if (!f || n_iterations < 0 || check_offsets(offsets, n_subsets) || (offsets[n_subsets] > offsets[0] && !events))
+        return fail(ctx, LMOSEM_EINVAL, "reconstruct_host: bad arguments");
+    // this rank's block of every subset: the only events it uploads (block distribution)
+    int64_t cap = 1;
+    for (int32_t l = 0; l < n_subsets; ++l) {
+        int64_t b, e;
+        block_range(offsets[l + 1] - offsets[l], ctx->rank, ctx->world, &b, &e);
+        cap = std::max(cap, e - b);
+    }
+    if (cap > ctx->dev_ev_cap) {
+        for (int k = 0; k < 2; ++k) {
+            if (ctx->dev_ev[k]) CK(cudaFree(ctx->dev_ev[k]));
+            ctx->dev_ev[k] = nullptr;
+        }
+        ctx->dev_ev_cap = 0;
+        for (int k = 0; k < 2; ++k) CK(cudaMalloc(&ctx->dev_ev[k], sizeof(lmosem_event) * cap));
+        ctx->dev_ev_cap = cap;
+    }
+    if (!ctx->dev_f) CK(cudaMalloc(&ctx->dev_f, sizeof(float) * ctx->V));
+    CK(cudaMemcpyAsync(ctx->dev_f, f, sizeof(float) * ctx->V, cudaMemcpyHostToDevice, ctx->stream));
+    // buffers start free
+    for (int k = 0; k < 2; ++k) CK(cudaEventRecord(ctx->ev_consumed[k], ctx->stream));
+    int64_t step = 0;
+    for (int32_t it = 0; it < n_iterations; ++it)
+        for (int32_t l = 0; l < n_subsets; ++l, ++step) {
+            const int k = (int)(step & 1);
+            int64_t b, e;
+            block_range(offsets[l + 1] - offsets[l], ctx->rank, ctx->world, &b, &e);
+            CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_consumed[k], 0));
+            cudaEvent_t h0 = nullptr, h1 = nullptr;
+            if (ctx->timing) {
+                for (int q = 0; q < 2; ++q) {
+                    if (ctx->h2d_pool.empty()) {
+                        cudaEvent_t ev;
+                        CK(cudaEventCreate(&ev));
+                        ctx->h2d_pool.push_back(ev);
+                    }
+                    (q ? h1 : h0) = ctx->h2d_pool.back();
+                    ctx->h2d_pool.pop_back();
+                }
+                CK(cudaEventRecord(h0, ctx->copy_stream));
+            }
+            if (e > b)
+                CK(cudaMemcpyAsync(ctx->dev_ev[k], events + offsets[l] + b, sizeof(lmosem_event) * (e - b),
+                                   cudaMemcpyHostToDevice, ctx->copy_stream));
+            if (ctx->timing) {
+                CK(cudaEventRecord(h1, ctx->copy_stream));
+                ctx->h2d_pending.push_back(h0);
+                ctx->h2d_pending.push_back(h1);
+            }
+            CK(cudaEventRecord(ctx->ev_copied[k], ctx->copy_stream));
+            CK(cudaStreamWaitEvent(ctx->stream, ctx->ev_copied[k], 0));
+            lmosem_status s = subset_iteration(ctx, ctx->dev_ev[k], e - b, ctx->dev_f, false);
+            if (s) return s;
+            CK(cudaEventRecord(ctx->ev_consumed[k], ctx->stream));
+        }
+    CK(cudaMemcpyAsync(f, ctx->dev_f, sizeof(float) * ctx->V, cudaMemcpyDeviceToHost, ctx->stream));
+    CK(cudaStreamSynchronize(ctx->stream));
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
+                                            const float* f, float* c_out) {
+    USABLE(ctx);
+    if (!f || !c_out || n_events < 0 || (n_events > 0 && !events))
+        return fail(ctx, LMOSEM_EINVAL, "error_image: bad arguments");
+    CK(cudaMemsetAsync(c_out, 0, sizeof(float) * ctx->V, ctx->stream));
+    return launch_project(ctx, events, n_events, f, c_out, nullptr, 0);
+}
+
+LMOSEM_API lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
+                                        const float* f, float* fp_out) {
+    USABLE(ctx);
+    if (!f || n_events < 0 || (n_events > 0 && (!events || !fp_out)))
+        return fail(ctx, LMOSEM_EINVAL, "forward: bad arguments");
+    return launch_project(ctx, events, n_events, f, nullptr, fp_out, 1);
+}
+
+LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {
+    USABLE(ctx);
+    if (!f || !c) return fail(ctx, LMOSEM_EINVAL, "update: bad arguments");
+    return launch_update(ctx, f, c);
+}
+
+LMOSEM_API lmosem_status lmosem_synchronize(lmosem_ctx* ctx) {
+    USABLE(ctx);
+    CK(cudaStreamSynchronize(ctx->stream));
+    CK(cudaStreamSynchronize(ctx->copy_stream));
+    if (ctx->world > 1 && ctx->comm) {
+        ncclResult_t async_err = ncclSuccess;
+        NK(ncclCommGetAsyncError(ctx->comm, &async_err));
+        if (async_err != ncclSuccess)
+            return fail(ctx, LMOSEM_ENCCL, std::string("nccl async: ") + ncclGetErrorString(async_err));
+    }
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_set_timing(lmosem_ctx* ctx, int32_t enable) {
+    USABLE(ctx);
+    lmosem_status s = resolve_timing(ctx);
+    if (s) return s;
+    ctx->timing = enable != 0;
+    if (ctx->timing) {
+        ctx->st.project_ms = ctx->st.combine_ms = ctx->st.update_ms = ctx->st.h2d_ms = 0.0;
+        ctx->st.timed_subsets = 0;
+    }
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_get_stats(lmosem_ctx* ctx, lmosem_stats* out) {
+    USABLE(ctx);
+    if (!out) return LMOSEM_EINVAL;
+    lmosem_status s = resolve_timing(ctx);
+    if (s) return s;
+    *out = ctx->st;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
+    if (!ctx) return LMOSEM_OK;
+    if (ctx->stream) cudaStreamSynchronize(ctx->stream);
+    if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
+    if (ctx->comm) ncclCommDestroy(ctx->comm);
+    for (auto& pm : ctx->pending)
+        for (int k = 0; k < 4; ++k) cudaEventDestroy(pm.e[k]);
+    for (auto& pm : ctx->pool)
+        for (int k = 0; k < 4; ++k) cudaEventDestroy(pm.e[k]);
+    for (auto e : ctx->h2d_pending) cudaEventDestroy(e);
+    for (auto e : ctx->h2d_pool) cudaEventDestroy(e);
+    for (int k = 0; k < 2; ++k) {
+        if (ctx->dev_ev[k]) cudaFree(ctx->dev_ev[k]);
+        if (ctx->ev_copied[k]) cudaEventDestroy(ctx->ev_copied[k]);
+        if (ctx->ev_consumed[k]) cudaEventDestroy(ctx->ev_consumed[k]);
+    }
+    if (ctx->dev_f) cudaFree(ctx->dev_f);
+    if (ctx->c) cudaFree(ctx->c);
+    if (ctx->norm) cudaFree(ctx->norm);
+    if (ctx->own_stream) cudaStreamDestroy(ctx->own_stream);
+    if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
+    delete ctx;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API const char* lmosem_last_error(const lmosem_ctx* ctx) {
+    if (!ctx) return g_init_err.empty() ? "lmosem: null context" : g_init_err.c_str();
+    return ctx->err.c_str();
+}

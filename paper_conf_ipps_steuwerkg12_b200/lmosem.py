@@ -1,0 +1,265 @@
+"""Thin Python binding of the C ABI in ``include/lmosem.h`` (argument marshalling only).
+
+Every step of the LM-OSEM subset iteration runs in ``liblmosem.so`` (sm_100a kernels +
+NCCL); this module only converts torch tensors / numpy arrays to pointers. PyTorch
+provides device memory, streams and the process group used to broadcast the NCCL id.
+There is no CPU fallback: without the CUDA library or a GPU every call raises.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+import numpy as np
+
+_PKG = os.path.dirname(os.path.abspath(__file__))
+SO_PATH = os.path.join(_PKG, "liblmosem.so")
+
+OK, EINVAL, ENOMEM, ECUDA, ENCCL, ESTATE = range(6)
+_NAMES = {0: "OK", 1: "EINVAL", 2: "ENOMEM", 3: "ECUDA", 4: "ENCCL", 5: "ESTATE"}
+NCCL_ID_BYTES = 128
+
+# every symbol include/lmosem.h declares (checked by tests/test_abi.py)
+EXPORTS = (
+    "lmosem_version", "lmosem_block_range", "lmosem_nccl_unique_id", "lmosem_init", "lmosem_set_stream",
+    "lmosem_subset_step", "lmosem_reconstruct", "lmosem_reconstruct_host", "lmosem_error_image",
+    "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
+    "lmosem_destroy", "lmosem_last_error",
+)
+
+
+class LmosemError(RuntimeError):
+    def __init__(self, status: int, msg: str):
+        super().__init__(f"lmosem {_NAMES.get(status, status)}: {msg}")
+        self.status = status
+
+
+class Dist(ctypes.Structure):
+    _fields_ = [("rank", ctypes.c_int32), ("world", ctypes.c_int32), ("nccl_unique_id", ctypes.c_void_p)]
+
+
+class Stats(ctypes.Structure):
+    _fields_ = [("launches", ctypes.c_int64), ("subsets", ctypes.c_int64), ("events", ctypes.c_int64),
+                ("timed_subsets", ctypes.c_int64), ("project_ms", ctypes.c_double),
+                ("combine_ms", ctypes.c_double), ("update_ms", ctypes.c_double), ("h2d_ms", ctypes.c_double)]
+
+    def as_dict(self) -> dict:
+        return {k: getattr(self, k) for k, _ in self._fields_}
+
+
+_lib = None
+_P = ctypes.c_void_p
+_I64 = ctypes.c_int64
+_I32 = ctypes.c_int32
+_S = ctypes.c_int
+
+
+def load(build_if_missing: bool = False) -> ctypes.CDLL:
+    """Loads liblmosem.so (fails loudly if it is missing; no fallback)."""
+    global _lib
+    if _lib is not None:
+        return _lib
+    if build_if_missing:
+        from . import build as _b
+        _b.build()
+    if not os.path.exists(SO_PATH):
+        raise ImportError(f"{SO_PATH} not built: run `python -c 'import __graft_entry__ as g; g.build()'`")
+    lib = ctypes.CDLL(SO_PATH)
+    sig = {
+        "lmosem_version": ([], ctypes.c_char_p),
+        "lmosem_block_range": ([_I64, _I32, _I32, ctypes.POINTER(_I64), ctypes.POINTER(_I64)], _S),
+        "lmosem_nccl_unique_id": ([_P, ctypes.c_size_t], _S),
+        "lmosem_init": ([ctypes.POINTER(_P), _P, _P, _P, ctypes.POINTER(Dist)], _S),
+        "lmosem_set_stream": ([_P, _P], _S),
+        "lmosem_subset_step": ([_P, _P, _I64, _P], _S),
+        "lmosem_reconstruct": ([_P, _P, _P, _I32, _I32, _P], _S),
+        "lmosem_reconstruct_host": ([_P, _P, _P, _I32, _I32, _P], _S),
+        "lmosem_error_image": ([_P, _P, _I64, _P, _P], _S),
+        "lmosem_forward": ([_P, _P, _I64, _P, _P], _S),
+        "lmosem_update": ([_P, _P, _P], _S),
+        "lmosem_synchronize": ([_P], _S),
+        "lmosem_set_timing": ([_P, _I32], _S),
+        "lmosem_get_stats": ([_P, ctypes.POINTER(Stats)], _S),
+        "lmosem_destroy": ([_P], _S),
+        "lmosem_last_error": ([_P], ctypes.c_char_p),
+    }
+    for name, (args, res) in sig.items():
+        fn = getattr(lib, name)
+        fn.argtypes = args
+        fn.restype = res
+    _lib = lib
+    return lib
+
+
+def version() -> str:
+    return load().lmosem_version().decode()
+
+
+def block_range(n: int, rank: int, world: int) -> tuple[int, int]:
+    """Block distribution of n events over world ranks."""
+    b, e = _I64(), _I64()
+    st = load().lmosem_block_range(int(n), int(rank), int(world), ctypes.byref(b), ctypes.byref(e))
+    if st != OK:
+        raise LmosemError(st, "block_range: bad arguments")
+    return b.value, e.value
+
+
+def nccl_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(NCCL_ID_BYTES)
+    st = load().lmosem_nccl_unique_id(buf, NCCL_ID_BYTES)
+    if st != OK:
+        raise LmosemError(st, "ncclGetUniqueId failed")
+    return buf.raw
+
+
+def _dev_ptr(t, dtype_name: str, numel: int | None = None) -> int:
+    import torch
+    if not isinstance(t, torch.Tensor) or not t.is_cuda:
+        raise TypeError("expected a CUDA torch.Tensor")
+    if str(t.dtype) != f"torch.{dtype_name}":
+        raise TypeError(f"expected {dtype_name}, got {t.dtype}")
+    if not t.is_contiguous():
+        raise ValueError("tensor must be contiguous")
+    if numel is not None and t.numel() != numel:
+        raise ValueError(f"expected {numel} elements, got {t.numel()}")
+    return t.data_ptr()
+
+
+def _host_ptr(a, numel: int | None = None) -> int:
+    import torch
+    if isinstance(a, torch.Tensor):
+        if a.is_cuda or a.dtype != torch.float32 or not a.is_contiguous():
+            raise TypeError("expected a contiguous float32 CPU tensor")
+        if numel is not None and a.numel() != numel:
+            raise ValueError(f"expected {numel} elements")
+        return a.data_ptr()
+    if not (isinstance(a, np.ndarray) and a.dtype == np.float32 and a.flags.c_contiguous):
+        raise TypeError("expected a contiguous float32 numpy array")
+    if numel is not None and a.size != numel:
+        raise ValueError(f"expected {numel} elements")
+    return a.ctypes.data
+
+
+class Reconstructor:
+    """One LM-OSEM context (one GPU / rank). See include/lmosem.h for semantics.
+
+    ``norm``: V float32 sensitivity image (CUDA tensor or host array), copied at init.
+    ``dist``: None for one GPU, or (rank, world, nccl_id_bytes) for a collective context.
+    ``stream``: torch.cuda.Stream to enqueue on (default: torch's current stream).
+    """
+
+    def __init__(self, dims, voxel_mm, norm, dist=None, stream=None):
+        import torch
+        lib = load()
+        if not torch.cuda.is_available():
+            raise RuntimeError("lmosem needs a CUDA device (no CPU fallback)")
+        self._lib = lib
+        self.dims = tuple(int(d) for d in dims)
+        self.voxel_mm = tuple(float(v) for v in voxel_mm)
+        self.V = self.dims[0] * self.dims[1] * self.dims[2]
+        d = (ctypes.c_int32 * 3)(*self.dims)
+        v = (ctypes.c_float * 3)(*self.voxel_mm)
+        if isinstance(norm, torch.Tensor) and norm.is_cuda:
+            nptr = _dev_ptr(norm, "float32", self.V)
+            torch.cuda.current_stream().synchronize()
+        else:
+            nptr = _host_ptr(norm, self.V)
+        self._keep = None
+        dptr = None
+        if dist is not None:
+            rank, world, uid = dist
+            self._keep = ctypes.create_string_buffer(bytes(uid), NCCL_ID_BYTES)
+            dptr = ctypes.byref(Dist(int(rank), int(world), ctypes.cast(self._keep, ctypes.c_void_p)))
+        h = _P()
+        st = lib.lmosem_init(ctypes.byref(h), d, v, nptr, dptr)
+        if st != OK:
+            raise LmosemError(st, lib.lmosem_last_error(None).decode())
+        self._h = h
+        self.rank, self.world = (0, 1) if dist is None else (int(dist[0]), int(dist[1]))
+        self.set_stream(stream if stream is not None else torch.cuda.current_stream())
+
+    # -- plumbing
+    def _check(self, st: int):
+        if st != OK:
+            raise LmosemError(st, self._lib.lmosem_last_error(self._h).decode())
+
+    def set_stream(self, stream):
+        self._stream = stream
+        self._check(self._lib.lmosem_set_stream(self._h, _P(stream.cuda_stream if stream is not None else 0)))
+
+    def close(self):
+        if getattr(self, "_h", None) is not None and self._h.value:
+            self._lib.lmosem_destroy(self._h)
+            self._h = _P()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.close()
+
+    # -- the path (device buffers; stream-ordered)
+    @staticmethod
+    def _events_ptr(events) -> tuple[int, int]:
+        n = events.numel() // 6 if events.numel() else 0
+        if events.numel() != 6 * n:
+            raise ValueError("events must hold 6 floats per event")
+        return (_dev_ptr(events, "float32") if n else 0), n
+
+    def subset_step(self, events, f):
+        """One subset iteration: step 1 (this rank's block), c all-reduce, step 2 on f."""
+        ep, n = self._events_ptr(events)
+        self._check(self._lib.lmosem_subset_step(self._h, ep, n, _dev_ptr(f, "float32", self.V)))
+
+    def reconstruct(self, events, offsets, n_iterations, f):
+        """n_iterations passes over subsets events[offsets[l]:offsets[l+1]] (in events)."""
+        ep, _ = self._events_ptr(events)
+        off = np.ascontiguousarray(offsets, dtype=np.int64)
+        self._check(self._lib.lmosem_reconstruct(self._h, ep, off.ctypes.data, off.size - 1, int(n_iterations),
+                                                 _dev_ptr(f, "float32", self.V)))
+
+    def reconstruct_host(self, events, offsets, n_iterations, f):
+        """Host events + host f (in/out); H2D streaming overlapped with projection."""
+        off = np.ascontiguousarray(offsets, dtype=np.int64)
+        self._check(self._lib.lmosem_reconstruct_host(self._h, _host_ptr(events), off.ctypes.data, off.size - 1,
+                                                      int(n_iterations), _host_ptr(f, self.V)))
+
+    def error_image(self, events, f, c_out):
+        ep, n = self._events_ptr(events)
+        self._check(self._lib.lmosem_error_image(self._h, ep, n, _dev_ptr(f, "float32", self.V),
+                                                 _dev_ptr(c_out, "float32", self.V)))
+
+    def forward(self, events, f, fp_out):
+        ep, n = self._events_ptr(events)
+        self._check(self._lib.lmosem_forward(self._h, ep, n, _dev_ptr(f, "float32", self.V),
+                                             _dev_ptr(fp_out, "float32", n) if n else 0))
+
+    def update(self, f, c):
+        self._check(self._lib.lmosem_update(self._h, _dev_ptr(f, "float32", self.V), _dev_ptr(c, "float32", self.V)))
+
+    def synchronize(self):
+        self._check(self._lib.lmosem_synchronize(self._h))
+
+    def set_timing(self, enable: bool):
+        self._check(self._lib.lmosem_set_timing(self._h, 1 if enable else 0))
+
+    def stats(self) -> dict:
+        s = Stats()
+        self._check(self._lib.lmosem_get_stats(self._h, ctypes.byref(s)))
+        return s.as_dict()
+
+
+def make_dist(rank: int, world: int, group=None) -> tuple[int, int, bytes] | None:
+    """NCCL id from rank 0, broadcast with torch.distributed (any backend)."""
+    if world <= 1:
+        return None
+    import torch.distributed as dist
+    obj = [nccl_unique_id() if rank == 0 else None]
+    dist.broadcast_object_list(obj, src=0, group=group)
+    return (rank, world, obj[0])

@@ -1,0 +1,312 @@
+"""GPU parity: the CUDA path (through the C ABI) against the float64 oracle.
+
+Acceptance (BASELINE.json north_star):
+  - after one subset: max |f_gpu - f_or| / f_or <= 1e-4 over voxels with f_or > 1e-3 max f_or;
+  - after a full reconstruction: ||f_gpu - f_or||_2 / ||f_or||_2 <= 1e-3.
+Only the ordering of fp32 atomics (and fp32 rounding) may differ.
+"""
+import numpy as np
+import pytest
+
+import lmgen
+import oracle
+from conftest import GOLDEN, read_golden_paths
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+MAXREL_SUBSET = 1e-4
+REL_L2_RECON = 1e-3
+
+
+@pytest.fixture(scope="module")
+def pkg():
+    if not torch.cuda.is_available():
+        pytest.skip("needs a GPU")
+    import paper_conf_ipps_steuwerkg12_b200 as p
+    p.load()
+    return p
+
+
+def dev(a):
+    return torch.from_numpy(np.ascontiguousarray(a)).cuda()
+
+
+def maxrel(got, ref):
+    m = ref > 1e-3 * ref.max()
+    return float(np.max(np.abs(got[m] - ref[m]) / ref[m]))
+
+
+def rel_l2(got, ref):
+    return float(np.linalg.norm(got - ref) / np.linalg.norm(ref))
+
+
+_cache = {}
+
+
+def inputs(name, n_events=None):
+    key = (name, n_events)
+    if key not in _cache:
+        cfg = lmgen.CONFIGS[name]
+        if n_events is not None:
+            cfg = lmgen.with_(cfg, n_events=n_events)
+        ev = lmgen.events(cfg, 0, cfg.n_events * cfg.n_subsets)
+        _cache[key] = (cfg, ev, lmgen.norm(cfg))
+    return _cache[key]
+
+
+def gpu_subset(pkg, cfg, ev, s, f0):
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f = dev(f0.astype(np.float32))
+    rec.subset_step(dev(ev), f)
+    rec.synchronize()
+    out = f.cpu().numpy().astype(np.float64)
+    rec.close()
+    return out
+
+
+# ------------------------------------------------------------------ golden / edge cases
+def test_golden_paths_on_gpu(pkg):
+    """Hand-derived paths (tests/golden/paths_4cube.txt), incl. corner/face ties: with
+    f = 1 the error image of one event is c_j = a_ij / sum_j a_ij, so c * chord = a_ij."""
+    rec = pkg.Reconstructor((4, 4, 4), (1, 1, 1), dev(np.ones(64, np.float32)))
+    f = dev(np.ones(64, np.float32))
+    for name, p1, p2, pairs in read_golden_paths():
+        ev = dev(np.array([p1 + p2], np.float32))
+        c = torch.empty(64, device="cuda")
+        rec.error_image(ev, f, c)
+        fp = torch.empty(1, device="cuda")
+        rec.forward(ev, f, fp)
+        c = c.cpu().numpy().astype(np.float64)
+        chord = sum(l for _, l in pairs)
+        assert abs(fp.item() - chord) <= 1e-5 * max(chord, 1), name
+        exp = np.zeros(64)
+        for j, l in pairs:
+            exp[j] = l / chord if chord > 0 else 0
+        np.testing.assert_allclose(c, exp, rtol=2e-6, atol=1e-7, err_msg=name)
+    rec.close()
+
+
+def test_golden_em_update_on_gpu(pkg):
+    cases = {c[0]: c for c in read_golden_paths()}
+    ev = np.array([cases["G1"][1] + cases["G1"][2], cases["G2"][1] + cases["G2"][2]], np.float32)
+    line = [l for l in open(f"{GOLDEN}/em_4cube.txt") if l.strip() and not l.startswith("#")][0]
+    exp = np.ones(64)
+    for tok in line.split():
+        j, v = tok.split(":")
+        exp[int(j)] = float(v)
+    got = gpu_subset(pkg, lmgen.with_(lmgen.CONFIGS["C1"], dims=(4, 4, 4), voxel_mm=(1, 1, 1)), ev,
+                     np.ones(64, np.float32), np.ones(64))
+    np.testing.assert_allclose(got, exp, rtol=1e-6)
+
+
+def test_degenerate_and_empty(pkg):
+    cfg = lmgen.CONFIGS["C1"]
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(np.ones(cfg.n_voxels, np.float32)))
+    f = dev(np.full(cfg.n_voxels, 2.0, np.float32))
+    nan = float("nan")
+    ev = np.array([[0, 0, 0, 0, 0, 0], [30, 30, 30, 40, 40, 40], [nan, 0, 0, 1, 1, 1],
+                   [0, 0, float("inf"), 1, 1, 1], [-20, 8, 0, 20, 8, 0]], np.float32)
+    rec.subset_step(dev(ev), f)
+    rec.subset_step(torch.empty(0, 6, device="cuda"), f)  # empty subset: f unchanged
+    rec.synchronize()
+    assert torch.all(f == 2.0).item()
+    rec.close()
+
+
+def test_axis_parallel_lors(pkg):
+    """LORs exactly parallel to one or two axes (zero direction components)."""
+    cfg = lmgen.CONFIGS["C1"]
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    rng = np.random.default_rng(0)
+    ev = []
+    for k in range(300):
+        p = rng.uniform(-7.9, 7.9, 3)
+        q = p.copy()
+        axes = [k % 3] if k % 2 else [k % 3, (k + 1) % 3]
+        for a in axes:
+            p[a], q[a] = -12.0, 12.0
+        ev.append(np.concatenate([p, q]))
+    ev = np.array(ev, np.float32)
+    f0 = rng.uniform(0.5, 2.0, cfg.n_voxels)
+    s = lmgen.norm(cfg)
+    got = gpu_subset(pkg, cfg, ev, s, f0)
+    ref = oracle.subset_step(g, ev, s, f0.astype(np.float32))
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+# ------------------------------------------------------------------ C1 (configs[0])
+def test_c1_forward_matches_oracle(pkg):
+    cfg, ev, s = inputs("C1")
+    rng = np.random.default_rng(1)
+    f0 = rng.uniform(0.5, 2.0, cfg.n_voxels).astype(np.float32)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    fp = torch.empty(len(ev), device="cuda")
+    rec.forward(dev(ev), dev(f0), fp)
+    rec.synchronize()
+    ref = oracle.forward(oracle.geom(cfg.dims, cfg.voxel_mm), ev, f0)
+    got = fp.cpu().numpy()
+    assert np.all((ref > 0) == (got > 0))
+    m = ref > 0
+    assert np.max(np.abs(got[m] - ref[m]) / ref[m]) <= 2e-6
+    rec.close()
+
+
+def test_c1_error_image_matches_oracle(pkg):
+    cfg, ev, s = inputs("C1")
+    f0 = np.random.default_rng(2).uniform(0.5, 2.0, cfg.n_voxels).astype(np.float32)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    c = torch.empty(cfg.n_voxels, device="cuda")
+    rec.error_image(dev(ev[:cfg.n_events]), dev(f0), c)
+    rec.synchronize()
+    ref = oracle.error_image(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], f0)
+    got = c.cpu().numpy()
+    assert np.all((ref > 0) == (got > 0))
+    m = ref > 1e-3 * ref.max()
+    assert np.max(np.abs(got[m] - ref[m]) / ref[m]) <= 1e-5
+    rec.close()
+
+
+def test_c1_one_subset(pkg):
+    cfg, ev, s = inputs("C1")
+    f0 = np.ones(cfg.n_voxels)
+    got = gpu_subset(pkg, cfg, ev[:cfg.n_events], s, f0)
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], s, f0)
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+def test_c1_listing2_literal_mode(pkg):
+    """s = 1: Listing 2 exactly (f_j *= c_j where c_j > 0)."""
+    cfg, ev, _ = inputs("C1")
+    s = np.ones(cfg.n_voxels, np.float32)
+    f0 = np.random.default_rng(3).uniform(0.5, 1.5, cfg.n_voxels)
+    got = gpu_subset(pkg, cfg, ev[:cfg.n_events], s, f0)
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], s, f0.astype(np.float32))
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+@pytest.mark.parametrize("iters", [1, 3])
+def test_c1_full_reconstruction(pkg, iters):
+    cfg, ev, s = inputs("C1")
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(dev(ev), off, iters, f)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, iters, s, np.ones(cfg.n_voxels))
+    assert rel_l2(got, ref) <= REL_L2_RECON
+    assert np.all(got > 0)
+    st = rec.stats()
+    assert st["subsets"] == iters * cfg.n_subsets and st["launches"] == 2 * iters * cfg.n_subsets
+    rec.close()
+
+
+def test_c1_host_reconstruct_matches_device(pkg):
+    cfg, ev, s = inputs("C1")
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    fd = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(dev(ev), off, 2, fd)
+    rec.synchronize()
+    fh = np.ones(cfg.n_voxels, np.float32)
+    evh = torch.from_numpy(ev).pin_memory()
+    rec.reconstruct_host(evh, off, 2, fh)
+    np.testing.assert_allclose(fh, fd.cpu().numpy(), rtol=1e-5)
+    rec.close()
+
+
+def test_emulated_psd_ranks(pkg):
+    """PAPER.md §IV.A (lines 476-485): summing the error images of the P blocks of a
+    subset (each computed separately, as P ranks would) equals the whole subset's."""
+    cfg, ev, s = inputs("C1")
+    ev = ev[:cfg.n_events]
+    f0 = dev(np.random.default_rng(4).uniform(0.5, 2, cfg.n_voxels).astype(np.float32))
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    whole = torch.empty(cfg.n_voxels, device="cuda")
+    rec.error_image(dev(ev), f0, whole)
+    for P in (2, 3, 8):
+        acc = torch.zeros(cfg.n_voxels, device="cuda", dtype=torch.float64)
+        for r in range(P):
+            b, e = pkg.block_range(len(ev), r, P)
+            part = torch.empty(cfg.n_voxels, device="cuda")
+            rec.error_image(dev(ev[b:e]), f0, part)
+            acc += part.double()
+        torch.testing.assert_close(acc.float(), whole, rtol=1e-5, atol=1e-9)
+    rec.close()
+
+
+def test_timing_stats(pkg):
+    cfg, ev, s = inputs("C1")
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.set_timing(True)
+    rec.subset_step(dev(ev[:cfg.n_events]), f)
+    st = rec.stats()
+    assert st["timed_subsets"] == 1 and st["project_ms"] > 0 and st["update_ms"] > 0
+    rec.close()
+
+
+# ------------------------------------------------------------------ paper-shaped configs
+@pytest.mark.parametrize("name", ["C2", "C5"])
+def test_one_subset_paper_shaped(pkg, name):
+    """One full 10^6-event subset (configs[1] / configs[4]) against the oracle."""
+    cfg = lmgen.CONFIGS[name]
+    ev = lmgen.subset_events(cfg, 0)
+    s = lmgen.norm(cfg)
+    f0 = np.ones(cfg.n_voxels)
+    got = gpu_subset(pkg, cfg, ev, s, f0)
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev, s, f0)
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+def test_c2_full_reconstruction(pkg):
+    """configs[1]: 10 subsets x 10^6 events, 1 iteration, relative L2 after the recon."""
+    cfg, ev, s = inputs("C2")
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(dev(ev), off, 1, f)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    rec.close()
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, np.ones(cfg.n_voxels))
+    assert rel_l2(got, ref) <= REL_L2_RECON
+    assert np.all(got > 0)
+
+
+def test_c4_full_size_properties(pkg):
+    """configs[3] at full size (300x300x560, 10^7 events in one subset): the oracle
+    checks sampled forward projections one by one; the back-projection is checked by
+    count conservation sum_{c>0} s f_new = N_eff, which holds at any size."""
+    cfg = lmgen.CONFIGS["C4"]
+    ev = lmgen.subset_events(cfg, 0)
+    s = lmgen.norm(cfg)
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f0 = np.ones(cfg.n_voxels, np.float32)
+    evd = dev(ev)
+    # sampled forward projections
+    idx = np.random.default_rng(5).choice(len(ev), 2000, replace=False)
+    fp = torch.empty(len(idx), device="cuda")
+    rec.forward(dev(ev[idx]), dev(f0), fp)
+    ref_fp = oracle.forward(g, ev[idx], f0)
+    m = ref_fp > 0
+    assert np.max(np.abs(fp.cpu().numpy()[m] - ref_fp[m]) / ref_fp[m]) <= 2e-6
+    # count conservation of the full subset (every C4 LOR passes through its emission
+    # point inside the phantom, so N_eff = N with f0 = 1)
+    assert np.all(ref_fp > 0)
+    f = dev(f0)
+    c = torch.empty(cfg.n_voxels, device="cuda")
+    rec.error_image(evd, f, c)
+    cs = c.cpu().numpy().astype(np.float64)
+    assert abs(cs.sum() - len(ev)) <= 1e-4 * len(ev)
+    rec.update(f, c)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    hit = cs > 0
+    total = float(np.sum(s.astype(np.float64)[hit] * got[hit]))
+    assert abs(total - len(ev)) <= 1e-4 * len(ev)
+    assert np.all(got > 0) and np.all(got[~hit] == 1.0)
+    assert torch.count_nonzero(c).item() == 0  # the update re-zeroes c
+    rec.close()
