@@ -106,8 +106,9 @@ lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
 lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
                           const float* norm, const lmosem_dist* dist);
 
-/* Uses the given cudaStream_t (as void*) for all later device work; NULL restores the
- * context's own stream. The stream must belong to the context's device. */
+/* Uses the given cudaStream_t (as void*) for all later device work; NULL means the CUDA
+ * default stream (torch's default stream is NULL). Until this is called the context uses
+ * its own non-blocking stream. The stream must belong to the context's device. */
 lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream);
 
 /* One subset iteration (step 1, combine, step 2) over n_events device events; f is the

@@ -290,7 +290,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
 
 LMOSEM_API lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream) {
     USABLE(ctx);
-    ctx->stream = stream ? (cudaStream_t)stream : ctx->own_stream;
+    ctx->stream = (cudaStream_t)stream;  // NULL = the CUDA default stream (e.g. torch's default)
     return LMOSEM_OK;
 }
 

@@ -185,7 +185,8 @@ class Reconstructor:
 
     def set_stream(self, stream):
         self._stream = stream
-        self._check(self._lib.lmosem_set_stream(self._h, _P(stream.cuda_stream if stream is not None else 0)))
+        # torch's default stream has handle 0 = the CUDA default stream for the library
+        self._check(self._lib.lmosem_set_stream(self._h, _P(stream.cuda_stream)))
 
     def close(self):
         if getattr(self, "_h", None) is not None and self._h.value:

@@ -1,0 +1,80 @@
+"""Multi-process (world size 2, gloo, CPU) tests of the N > 1 host logic.
+
+The GPU path's distribution (§IV.A) is: every rank
+gets the whole subset, projects its block [floor(rN/P), floor((r+1)N/P)) (block
+distribution, via the C ABI's lmosem_block_range), the per-rank error images are summed
+by an all-reduce (copy(add)), and every rank applies the update to its replica. Here the
+per-rank step 1 is the oracle and the all-reduce is gloo, so the decomposition and the
+NCCL-id broadcast plumbing are checked without a GPU.
+"""
+import os
+import socket
+
+import numpy as np
+import pytest
+
+torch = pytest.importorskip("torch")
+import torch.distributed as dist  # noqa: E402
+import torch.multiprocessing as mp  # noqa: E402
+
+
+def _free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def _worker(rank, world, port, q):
+    import sys
+    sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import lmgen
+        import oracle
+        import paper_conf_ipps_steuwerkg12_b200 as pkg
+        oracle.set_threads(2)
+        cfg = lmgen.CONFIGS["C1"]
+        g = oracle.geom(cfg.dims, cfg.voxel_mm)
+        ev = lmgen.subset_events(cfg, 0)
+        s = lmgen.norm(cfg)
+        f0 = np.random.default_rng(7).uniform(0.5, 2.0, cfg.n_voxels)
+        # block distribution through the C ABI (host-only entry point)
+        b, e = pkg.block_range(len(ev), rank, world)
+        c = torch.from_numpy(oracle.error_image(g, ev[b:e], f0))
+        dist.all_reduce(c)  # copy(add) combine
+        f_dist = oracle.update(f0, c.numpy(), s)
+        # every rank holds the same replica afterwards
+        gathered = [torch.empty_like(c) for _ in range(world)]
+        dist.all_gather(gathered, torch.from_numpy(f_dist))
+        same = all(torch.equal(gathered[0], x) for x in gathered)
+        f_one = oracle.subset_step(g, ev, s, f0)
+        err = float(np.max(np.abs(f_dist - f_one) / f_one))
+        # NCCL-id broadcast plumbing used by the GPU path
+        d = pkg.make_dist(rank, world)
+        ids = [None] * world
+        dist.all_gather_object(ids, d[2])
+        q.put((rank, b, e, same, err, d[0], d[1], len(d[2]), all(x == ids[0] for x in ids)))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_psd_two_ranks_gloo():
+    world = 2
+    port = _free_port()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = sorted(q.get(timeout=240) for _ in range(world))
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    (r0, b0, e0, same0, err0, *d0), (r1, b1, e1, same1, err1, *d1) = res
+    assert (b0, e0, b1, e1) == (0, 5000, 5000, 10000)
+    assert same0 and same1
+    assert err0 <= 1e-12 and err1 <= 1e-12
+    assert d0[:3] == [0, 2, 128] and d1[:3] == [1, 2, 128] and d0[3] and d1[3]
