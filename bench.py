@@ -241,10 +241,11 @@ def main():
     rec.set_timing(False)
     step_ms = [a.elapsed_time(b) for a, b in zip(starts, ends)]
     tot_ms = sum(step_ms)
-    t = torch.tensor([tot_ms, st["project_ms"], st["combine_ms"], st["update_ms"]], device=dev, dtype=torch.float64)
+    t = torch.tensor([tot_ms, st["convert_ms"], st["project_ms"], st["combine_ms"], st["update_ms"]], device=dev,
+                     dtype=torch.float64)
     if world > 1:
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
-    tot_ms, proj_ms, comb_ms, upd_ms = (float(x) for x in t.tolist())
+    tot_ms, conv_ms, proj_ms, comb_ms, upd_ms = (float(x) for x in t.tolist())
     K = args.steps
     value = N * K / (tot_ms * 1e-3)  # events of the whole job (each subset's N split over ranks)
 
@@ -301,9 +302,9 @@ def main():
     hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0) / proj_avg_s / 1e9, "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
     hbm["frac"] = hbm["achieved"] / hbm["peak"]
-    upd_bytes = 20.0 * cfg.n_voxels  # read f, c, s; write f, c
+    upd_bytes = 24.0 * cfg.n_voxels  # read f, c, s; write f (bricks), c; write f (caller layout)
     upd = {"bound": "hbm", "achieved": upd_bytes / (upd_ms / K * 1e-3) / 1e9, "peak": peaks["hbm_gbs"],
-           "unit": "GB/s", "peak_kind": peak_kind, "what": "k_update (20 B/voxel)"}
+           "unit": "GB/s", "peak_kind": peak_kind, "what": "k_update (24 B/voxel)"}
     upd["frac"] = upd["achieved"] / upd["peak"]
 
     line = {
@@ -315,7 +316,8 @@ def main():
                    "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block, f copy, c allreduce)",
                    "l2": "flushed before every timed step (256 MB write outside the step events)"},
         "s_per_recon": tot_ms / K * L * 1e-3, "s_per_recon_e2e": s_recon,
-        "phase_ms_per_step": {"project": proj_ms / K, "combine": comb_ms / K, "update": upd_ms / K},
+        "phase_ms_per_step": {"convert_f": conv_ms / K, "project": proj_ms / K, "combine": comb_ms / K,
+                              "update": upd_ms / K},
         "roofline": roof, "roofline_hbm_events": hbm, "roofline_update": upd,
         "gpu_launches": int(st["launches"] - launches0),
         "clocks": clk.summary(), "wall_s_timed_region": t_wall,

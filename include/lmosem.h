@@ -80,6 +80,7 @@ typedef struct {
     int64_t subsets;       /* subset iterations completed (all time) */
     int64_t events;        /* events projected by this rank (all time) */
     int64_t timed_subsets; /* subsets covered by the phase times below */
+    double convert_ms;     /* f -> internal brick layout (subset_step; first subset of reconstruct) */
     double project_ms;     /* step 1: fused traversal + forward + back-projection kernel */
     double combine_ms;     /* c all-reduce (world > 1) */
     double update_ms;      /* step 2: update kernel (also re-zeroes c) */
@@ -139,7 +140,7 @@ lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* events, int64_
                              const float* f, float* fp_out);
 
 /* Step 2 only, for tests: f_j <- f_j*c_j/s_j where c_j > 0 and s_j > 0 (device f and c,
- * the context's norm); c is re-zeroed. */
+ * both V float32 x-fastest; the context's norm); c is re-zeroed. */
 lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c);
 
 /* Waits for all work enqueued by this context. Reports asynchronous kernel faults. */

@@ -21,7 +21,7 @@ namespace {
 thread_local std::string g_init_err;  // message of the last failed lmosem_init on this thread
 
 struct PhaseMarks {
-    cudaEvent_t e[4];  // start, after project, after combine, after update
+    cudaEvent_t e[5];  // start, after f->brick conversion, after project, after combine, after update
 };
 
 }  // namespace
@@ -32,8 +32,15 @@ struct lmosem_ctx {
     float vox[3] = {0, 0, 0};
     int64_t V = 0;
     lmk::GridGeom geom{};
-    float* c = nullptr;     // error image (kept all-zero between subsets)
-    float* norm = nullptr;  // copy of s
+    lmk::BrickIt bricks{};
+    int64_t nbf = 0;           // floats per padded brick image (8 * bricks)
+    float* c = nullptr;        // error image, bricks (kept all-zero between subsets)
+    float* fb = nullptr;       // brick copy of the current f
+    float* norm = nullptr;     // s in bricks (halo = 0)
+    int* tab = nullptr;        // per-axis brick index tables (device)
+    float* scratch = nullptr;  // V floats, row layout (norm upload)
+    int cap = 0;               // path-piece capacity per warp
+    size_t proj_smem = 0;      // dynamic shared memory of k_project
     cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
     int rank = 0, world = 1;
     ncclComm_t comm = nullptr;
@@ -88,8 +95,27 @@ void block_range(int64_t n, int r, int P, int64_t* b, int64_t* e) {
     *e = (int64_t)((__int128)n * (r + 1) / P);
 }
 
-lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, const float* f, float* c,
-                             float* fp_out, int mode) {
+int grid_for(lmosem_ctx* ctx, int64_t items) {
+    const int64_t cap = (int64_t)ctx->num_sms * 16;
+    return (int)std::max<int64_t>(1, std::min<int64_t>((items + 255) / 256, cap));
+}
+
+lmosem_status launch_to_brick(lmosem_ctx* ctx, const float* row, float* br) {
+    lmk::k_row_to_brick<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(row, br, ctx->geom, ctx->bricks);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return LMOSEM_OK;
+}
+
+lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
+    lmk::k_brick_to_row<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(br, row, ctx->geom, ctx->bricks, zero);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return LMOSEM_OK;
+}
+
+// k_project over n device events against ctx->fb; mode 0 accumulates into ctx->c.
+lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* fp_out, int mode) {
     if (n <= 0) return LMOSEM_OK;
     const int64_t warps_needed = (n + 31) / 32;
     const int64_t blocks_needed = (warps_needed + 7) / 8;
@@ -97,17 +123,20 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
     const float* evf = reinterpret_cast<const float*>(ev);
     if (mode == 0)
-        lmk::k_project<0><<<grid, 256, 0, ctx->stream>>>(evf, n, f, c, nullptr, ctx->geom);
+        lmk::k_project<0><<<grid, 256, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, ctx->c, nullptr, ctx->tab,
+                                                                      ctx->geom, ctx->cap);
     else
-        lmk::k_project<1><<<grid, 256, 0, ctx->stream>>>(evf, n, f, nullptr, fp_out, ctx->geom);
+        lmk::k_project<1><<<grid, 256, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, nullptr, fp_out, ctx->tab,
+                                                                      ctx->geom, ctx->cap);
     CK(cudaGetLastError());
     ctx->st.launches++;
     return LMOSEM_OK;
 }
 
-lmosem_status launch_update(lmosem_ctx* ctx, float* f, float* c) {
-    const int vec = ((((uintptr_t)f) | ((uintptr_t)c) | ((uintptr_t)ctx->norm)) & 15) == 0;
-    lmk::k_update<<<ctx->upd_blocks, 256, 0, ctx->stream>>>(f, c, ctx->norm, ctx->V, vec);
+// step 2 on the bricks; f_row (caller layout) is written when non-null
+lmosem_status launch_update(lmosem_ctx* ctx, float* f_row) {
+    lmk::k_update<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->fb, ctx->c, ctx->norm, f_row, ctx->geom,
+                                                                          ctx->bricks);
     CK(cudaGetLastError());
     ctx->st.launches++;
     return LMOSEM_OK;
@@ -123,7 +152,7 @@ lmosem_status get_marks(lmosem_ctx* ctx, PhaseMarks** out) {
     if (!ctx->timing) return LMOSEM_OK;
     if (ctx->pool.empty()) {
         PhaseMarks pm;
-        for (int k = 0; k < 4; ++k) CK(cudaEventCreate(&pm.e[k]));
+        for (int k = 0; k < 5; ++k) CK(cudaEventCreate(&pm.e[k]));
         ctx->pool.push_back(pm);
     }
     ctx->pending.push_back(ctx->pool.back());
@@ -134,19 +163,23 @@ lmosem_status get_marks(lmosem_ctx* ctx, PhaseMarks** out) {
 
 // One subset iteration on the context's stream: this rank's block of step 1, the c
 // all-reduce (copy(add) -> every rank has the sum), step 2 on the full replica.
-lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* f, bool whole_subset) {
+// to_brick: refresh ctx->fb from f first; write_f: write the updated f to the caller.
+lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* f, bool whole_subset,
+                               bool to_brick, bool write_f) {
     int64_t b = 0, e = n;
     if (whole_subset) block_range(n, ctx->rank, ctx->world, &b, &e);
     PhaseMarks* pm = nullptr;
     lmosem_status s;
     if ((s = get_marks(ctx, &pm))) return s;
     if ((s = mark(ctx, pm, 0))) return s;
-    if ((s = launch_project(ctx, ev + b, e - b, f, ctx->c, nullptr, 0))) return s;
+    if (to_brick && (s = launch_to_brick(ctx, f, ctx->fb))) return s;
     if ((s = mark(ctx, pm, 1))) return s;
-    if (ctx->world > 1) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->V, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    if ((s = launch_project(ctx, ev + b, e - b, nullptr, 0))) return s;
     if ((s = mark(ctx, pm, 2))) return s;
-    if ((s = launch_update(ctx, f, ctx->c))) return s;
+    if (ctx->world > 1) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
     if ((s = mark(ctx, pm, 3))) return s;
+    if ((s = launch_update(ctx, write_f ? f : nullptr))) return s;
+    if ((s = mark(ctx, pm, 4))) return s;
     ctx->st.subsets++;
     ctx->st.events += e - b;
     return LMOSEM_OK;
@@ -162,14 +195,13 @@ lmosem_status check_offsets(const int64_t* off, int32_t L) {
 
 lmosem_status resolve_timing(lmosem_ctx* ctx) {
     for (auto& pm : ctx->pending) {
-        CK(cudaEventSynchronize(pm.e[3]));
-        float t01, t12, t23;
-        CK(cudaEventElapsedTime(&t01, pm.e[0], pm.e[1]));
-        CK(cudaEventElapsedTime(&t12, pm.e[1], pm.e[2]));
-        CK(cudaEventElapsedTime(&t23, pm.e[2], pm.e[3]));
-        ctx->st.project_ms += t01;
-        ctx->st.combine_ms += t12;
-        ctx->st.update_ms += t23;
+        CK(cudaEventSynchronize(pm.e[4]));
+        float t[4];
+        for (int k = 0; k < 4; ++k) CK(cudaEventElapsedTime(&t[k], pm.e[k], pm.e[k + 1]));
+        ctx->st.convert_ms += t[0];
+        ctx->st.project_ms += t[1];
+        ctx->st.combine_ms += t[2];
+        ctx->st.update_ms += t[3];
         ctx->st.timed_subsets++;
         ctx->pool.push_back(pm);
     }
@@ -188,7 +220,7 @@ lmosem_status resolve_timing(lmosem_ctx* ctx) {
 
 }  // namespace
 
-LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.1 sm_100a"; }
+LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.2 sm_100a"; }
 
 LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end) {
     if (!begin || !end || n < 0 || world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
@@ -240,9 +272,30 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         ctx->geom.lo[k] = -0.5 * (double)dims[k] * (double)voxel_mm[k];
         ctx->geom.inv_v[k] = 1.0 / (double)voxel_mm[k];
     }
-    ctx->geom.stride[0] = 1;
-    ctx->geom.stride[1] = dims[0];
-    ctx->geom.stride[2] = dims[0] * dims[1];
+    // padded brick layout: halo of HALO_LO below, >= 2 above, even extents
+    for (int k = 0; k < 3; ++k) ctx->geom.P[k] = (dims[k] + 4 + 1) & ~1;
+    ctx->geom.toff[0] = 0;
+    ctx->geom.toff[1] = ctx->geom.P[0];
+    ctx->geom.toff[2] = ctx->geom.P[0] + ctx->geom.P[1];
+    ctx->geom.tsize = ctx->geom.P[0] + ctx->geom.P[1] + ctx->geom.P[2];
+    ctx->bricks.BX = ctx->geom.P[0] / 2;
+    ctx->bricks.BY = ctx->geom.P[1] / 2;
+    ctx->bricks.BZ = ctx->geom.P[2] / 2;
+    ctx->bricks.nb = (int64_t)ctx->bricks.BX * ctx->bricks.BY * ctx->bricks.BZ;
+    ctx->nbf = 8 * ctx->bricks.nb;
+    if (ctx->nbf >= (int64_t(1) << 31)) {
+        delete ctx;
+        return LMOSEM_EINVAL;
+    }
+    std::vector<int> tab(ctx->geom.tsize);
+    {
+        const int64_t M[3] = {8, 8LL * ctx->bricks.BX, 8LL * ctx->bricks.BX * ctx->bricks.BY};
+        const int m[3] = {1, 2, 4};
+        for (int k = 0; k < 3; ++k)
+            for (int p = 0; p < ctx->geom.P[k]; ++p) tab[ctx->geom.toff[k] + p] = (int)(M[k] * (p >> 1) + m[k] * (p & 1));
+    }
+    ctx->cap = 3 * std::max(dims[0], std::max(dims[1], dims[2])) + 8;
+    ctx->proj_smem = sizeof(int) * (size_t)((ctx->geom.tsize + 1) & ~1) + 8 * sizeof(int2) * (size_t)ctx->cap;
 
     lmosem_status s = LMOSEM_OK;
     auto cuda = [&](cudaError_t e, const char* what) {
@@ -256,22 +309,42 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cudaDeviceProp prop;
     if (!cuda(cudaGetDeviceProperties(&prop, ctx->device), "cudaGetDeviceProperties")) return bail(s);
     ctx->num_sms = prop.multiProcessorCount;
-    cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, 256, 0),
+    if (ctx->proj_smem > (size_t)prop.sharedMemPerBlockOptin) {
+        ctx->err = "volume too large for the shared-memory path buffer";
+        return bail(LMOSEM_EINVAL);
+    }
+    cuda(cudaFuncSetAttribute(lmk::k_project<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
+         "smem attr");
+    cuda(cudaFuncSetAttribute(lmk::k_project<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
+         "smem attr");
+    cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, 256,
+                                                       ctx->proj_smem),
          "occupancy");
     if (ctx->proj_blocks_per_sm < 1) ctx->proj_blocks_per_sm = 1;
     ctx->upd_blocks = ctx->num_sms * 8;
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     ctx->stream = ctx->own_stream;
-    cuda(cudaMalloc(&ctx->c, sizeof(float) * V), "cudaMalloc(c)");
-    cuda(cudaMalloc(&ctx->norm, sizeof(float) * V), "cudaMalloc(norm)");
+    cuda(cudaMalloc(&ctx->c, sizeof(float) * ctx->nbf), "cudaMalloc(c)");
+    cuda(cudaMalloc(&ctx->fb, sizeof(float) * ctx->nbf), "cudaMalloc(fb)");
+    cuda(cudaMalloc(&ctx->norm, sizeof(float) * ctx->nbf), "cudaMalloc(norm)");
+    cuda(cudaMalloc(&ctx->scratch, sizeof(float) * V), "cudaMalloc(scratch)");
+    cuda(cudaMalloc(&ctx->tab, sizeof(int) * tab.size()), "cudaMalloc(tab)");
     for (int k = 0; k < 2; ++k) {
         cuda(cudaEventCreateWithFlags(&ctx->ev_copied[k], cudaEventDisableTiming), "cudaEventCreate");
         cuda(cudaEventCreateWithFlags(&ctx->ev_consumed[k], cudaEventDisableTiming), "cudaEventCreate");
     }
     if (s != LMOSEM_OK) return bail(s);
-    cuda(cudaMemcpyAsync(ctx->norm, norm, sizeof(float) * V, cudaMemcpyDefault, ctx->stream), "copy norm");
-    cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * V, ctx->stream), "memset c");
+    cuda(cudaMemcpyAsync(ctx->tab, tab.data(), sizeof(int) * tab.size(), cudaMemcpyHostToDevice, ctx->stream),
+         "copy tab");
+    cuda(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * V, cudaMemcpyDefault, ctx->stream), "copy norm");
+    cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * ctx->nbf, ctx->stream), "memset c");
+    cuda(cudaMemsetAsync(ctx->fb, 0, sizeof(float) * ctx->nbf, ctx->stream), "memset fb");
+    if (s == LMOSEM_OK) {
+        lmk::k_row_to_brick<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->scratch, ctx->norm,
+                                                                                     ctx->geom, ctx->bricks);
+        cuda(cudaGetLastError(), "k_row_to_brick(norm)");
+    }
     cuda(cudaStreamSynchronize(ctx->stream), "sync");
     if (s != LMOSEM_OK) return bail(s);
     if (world > 1) {
@@ -297,7 +370,7 @@ LMOSEM_API lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream) {
 LMOSEM_API lmosem_status lmosem_subset_step(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events, float* f) {
     USABLE(ctx);
     if (!f || n_events < 0 || (n_events > 0 && !events)) return fail(ctx, LMOSEM_EINVAL, "subset_step: bad arguments");
-    return subset_iteration(ctx, events, n_events, f, true);
+    return subset_iteration(ctx, events, n_events, f, true, true, true);
 }
 
 LMOSEM_API lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
@@ -305,9 +378,12 @@ LMOSEM_API lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event*
     USABLE(ctx);
     if (!f || n_iterations < 0 || check_offsets(offsets, n_subsets) || (offsets[n_subsets] > offsets[0] && !events))
         return fail(ctx, LMOSEM_EINVAL, "reconstruct: bad arguments");
+    const int64_t total = (int64_t)n_iterations * n_subsets;
+    int64_t step = 0;
     for (int32_t it = 0; it < n_iterations; ++it)
-        for (int32_t l = 0; l < n_subsets; ++l) {
-            lmosem_status s = subset_iteration(ctx, events + offsets[l], offsets[l + 1] - offsets[l], f, true);
+        for (int32_t l = 0; l < n_subsets; ++l, ++step) {
+            lmosem_status s = subset_iteration(ctx, events + offsets[l], offsets[l + 1] - offsets[l], f, true,
+                                               step == 0, step == total - 1);
             if (s) return s;
         }
     return LMOSEM_OK;
@@ -339,6 +415,7 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
     // buffers start free
     for (int k = 0; k < 2; ++k) CK(cudaEventRecord(ctx->ev_consumed[k], ctx->stream));
     int64_t step = 0;
+    const int64_t total = (int64_t)n_iterations * n_subsets;
     for (int32_t it = 0; it < n_iterations; ++it)
         for (int32_t l = 0; l < n_subsets; ++l, ++step) {
             const int k = (int)(step & 1);
@@ -368,7 +445,8 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
             }
             CK(cudaEventRecord(ctx->ev_copied[k], ctx->copy_stream));
             CK(cudaStreamWaitEvent(ctx->stream, ctx->ev_copied[k], 0));
-            lmosem_status s = subset_iteration(ctx, ctx->dev_ev[k], e - b, ctx->dev_f, false);
+            lmosem_status s = subset_iteration(ctx, ctx->dev_ev[k], e - b, ctx->dev_f, false, step == 0,
+                                               step == total - 1);
             if (s) return s;
             CK(cudaEventRecord(ctx->ev_consumed[k], ctx->stream));
         }
@@ -382,8 +460,10 @@ LMOSEM_API lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event*
     USABLE(ctx);
     if (!f || !c_out || n_events < 0 || (n_events > 0 && !events))
         return fail(ctx, LMOSEM_EINVAL, "error_image: bad arguments");
-    CK(cudaMemsetAsync(c_out, 0, sizeof(float) * ctx->V, ctx->stream));
-    return launch_project(ctx, events, n_events, f, c_out, nullptr, 0);
+    lmosem_status s;
+    if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
+    if ((s = launch_project(ctx, events, n_events, nullptr, 0))) return s;
+    return launch_to_row(ctx, ctx->c, c_out, 1);  // c_out <- c, c <- 0
 }
 
 LMOSEM_API lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
@@ -391,13 +471,20 @@ LMOSEM_API lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* eve
     USABLE(ctx);
     if (!f || n_events < 0 || (n_events > 0 && (!events || !fp_out)))
         return fail(ctx, LMOSEM_EINVAL, "forward: bad arguments");
-    return launch_project(ctx, events, n_events, f, nullptr, fp_out, 1);
+    lmosem_status s;
+    if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
+    return launch_project(ctx, events, n_events, fp_out, 1);
 }
 
 LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {
     USABLE(ctx);
     if (!f || !c) return fail(ctx, LMOSEM_EINVAL, "update: bad arguments");
-    return launch_update(ctx, f, c);
+    lmosem_status s;
+    if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
+    if ((s = launch_to_brick(ctx, c, ctx->c))) return s;
+    if ((s = launch_update(ctx, f))) return s;  // also re-zeroes the context's c
+    CK(cudaMemsetAsync(c, 0, sizeof(float) * ctx->V, ctx->stream));
+    return LMOSEM_OK;
 }
 
 LMOSEM_API lmosem_status lmosem_synchronize(lmosem_ctx* ctx) {
@@ -419,7 +506,7 @@ LMOSEM_API lmosem_status lmosem_set_timing(lmosem_ctx* ctx, int32_t enable) {
     if (s) return s;
     ctx->timing = enable != 0;
     if (ctx->timing) {
-        ctx->st.project_ms = ctx->st.combine_ms = ctx->st.update_ms = ctx->st.h2d_ms = 0.0;
+        ctx->st.convert_ms = ctx->st.project_ms = ctx->st.combine_ms = ctx->st.update_ms = ctx->st.h2d_ms = 0.0;
         ctx->st.timed_subsets = 0;
     }
     return LMOSEM_OK;
@@ -440,9 +527,9 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     for (auto& pm : ctx->pending)
-        for (int k = 0; k < 4; ++k) cudaEventDestroy(pm.e[k]);
+        for (int k = 0; k < 5; ++k) cudaEventDestroy(pm.e[k]);
     for (auto& pm : ctx->pool)
-        for (int k = 0; k < 4; ++k) cudaEventDestroy(pm.e[k]);
+        for (int k = 0; k < 5; ++k) cudaEventDestroy(pm.e[k]);
     for (auto e : ctx->h2d_pending) cudaEventDestroy(e);
     for (auto e : ctx->h2d_pool) cudaEventDestroy(e);
     for (int k = 0; k < 2; ++k) {
@@ -452,7 +539,10 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     }
     if (ctx->dev_f) cudaFree(ctx->dev_f);
     if (ctx->c) cudaFree(ctx->c);
+    if (ctx->fb) cudaFree(ctx->fb);
     if (ctx->norm) cudaFree(ctx->norm);
+    if (ctx->scratch) cudaFree(ctx->scratch);
+    if (ctx->tab) cudaFree(ctx->tab);
     if (ctx->own_stream) cudaStreamDestroy(ctx->own_stream);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     delete ctx;

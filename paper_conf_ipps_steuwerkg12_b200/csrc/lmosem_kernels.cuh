@@ -1,21 +1,29 @@
 // lmosem_kernels.cuh — sm_100a kernels of the LM-OSEM subset iteration.
 //
-// Step 1 (Listing 2 lines 5-13) is ONE fused kernel per subset: every warp
-// owns one line of response (LOR) at a time and walks it as a set of independent slabs
-// of its dominant axis:
-//   - per LOR, in float64: clip to the volume, pick the dominant axis a (largest
-//     |du_a| in voxel units), the minor-axis positions at the first slab plane and the
-//     slopes du_b/du_a, du_c/du_a (|slope| <= 1);
-//   - per slab i (lane k handles slabs k, k+32, ...): because |slope| <= 1 each minor
-//     axis crosses at most one voxel plane inside the slab, so the slab holds at most
-//     three path pieces; the minor position at the slab plane is one float64 FMA, and
-//     the crossing points are computed in float32 relative to that plane (all values in
-//     [0,1], so absolute error ~1e-7 voxel, independent of where the slab lies);
-//   - pass 1 gathers f along the pieces (forward projection, Listing 2 lines 9-10),
-//     a warp reduction gives fp; pass 2 recomputes the pieces and issues fp32
-//     red.global.add of len/fp into c (back-projection, lines 12-13). c (25 MB at the
-//     paper's 150x150x280) stays resident in the 126 MB L2.
-// Step 2 (lines 16-17 + norm) is a vectorised streaming kernel that also re-zeroes c.
+// Step 1 (Listing 2 lines 5-13) is ONE fused kernel per subset, k_project: a
+// warp owns one line of response (LOR) at a time:
+//   - setup, per LOR in float64 (one lane per event of a 32-event batch, broadcast by
+//     shuffles): clip to the volume, dominant axis a (largest |du_a| in voxel units),
+//     minor-axis positions at the first slab plane and slopes du_b/du_a, du_c/du_a
+//     (|slope| <= 1);
+//   - pass 1 (geometry): lane k takes slabs k, k+32, ... of the dominant axis. Each minor
+//     axis crosses at most one plane inside a slab, so a slab holds <= 3 pieces; the
+//     minor positions at the slab plane are one float64 FMA and the crossings are float32
+//     relative to that plane (values in [0,1], ~1e-7 voxel absolute error wherever the
+//     slab lies). The pieces (j, len) are compacted into the warp's shared-memory path
+//     buffer, slab-major;
+//   - pass 2 (forward projection, lines 9-10): lane m reads piece m and gathers f — lanes
+//     hold consecutive pieces of one path, so they share 32-byte sectors of the brick
+//     layout below; warp reduction gives fp;
+//   - pass 3 (back-projection, lines 12-13): lane m issues red.global.add.f32 of
+//     len/fp into c, again sector-coalesced. c stays resident in the 126 MB L2.
+// Internal image layout ("bricks"): the volume is padded by a halo (2 voxels low, >= 2
+// high, even extents) and stored as 2x2x2 bricks of 8 floats = one 32-byte L2 sector;
+// index J = Tx[px] + Ty[py] + Tz[pz] with T_axis(p) = M_axis*(p>>1) + m_axis*(p&1),
+// (M, m) = (8, 1), (8*BX, 2), (8*BX*BY, 4). Rounding slivers that step one voxel past
+// the volume land in the halo (f = 0 there, c ignored), so the hot loop has no range
+// checks. Step 2 (lines 16-17 + norm) is k_update over bricks; it also re-zeroes c and
+// writes the caller's x-fastest f.
 #pragma once
 #include <cuda_runtime.h>
 #include <math_constants.h>
@@ -23,27 +31,29 @@
 
 namespace lmk {
 
+constexpr int HALO_LO = 2;  // padded coordinate p = i + HALO_LO
+
 struct GridGeom {
-    int n[3];          // nx, ny, nz
-    int stride[3];     // 1, nx, nx*ny
-    double lo[3];      // volume lower corner (mm): -n*v/2
-    double inv_v[3];   // 1 / voxel size (1/mm)
+    int n[3];         // nx, ny, nz (real volume)
+    int P[3];         // padded extents (even, >= n + 4)
+    int toff[3];      // offsets of the per-axis index tables in the table array
+    int tsize;        // total table entries = P[0] + P[1] + P[2]
+    double lo[3];     // volume lower corner (mm): -n*v/2
+    double inv_v[3];  // 1 / voxel size (1/mm)
 };
 
-// Per-LOR traversal state, 21 x 32-bit words (broadcast lane -> warp by shuffles).
+// Per-LOR traversal state (broadcast lane -> warp by shuffles).
 struct Lor {
-    double wb0, wc0;   // minor-axis positions (voxel units) at the plane u_a = i0
-    double sb, sc;     // du_b/du_a, du_c/du_a
-    float isb, isc;    // 1/|sb|, 1/|sc| (+inf when the slope is 0)
-    float lunit;       // mm of chord per unit of u_a
-    float fin, fout;   // clip inside the first / last slab (local coordinate in [0,1])
-    int i0, ns;        // first slab index along a, number of slabs
-    int sa, sbs, scs;  // linear strides of axes a, b, c
-    int nb, nc;        // extents of axes b, c
-    int steps;         // bit0/1: sb >0/<0, bit2/3: sc >0/<0
+    double wb0, wc0;  // minor-axis positions (voxel units) at the plane u_a = i0
+    double sb, sc;    // du_b/du_a, du_c/du_a
+    float ab, bb, ac, bc;  // crossing position in a slab: d = fma(frac, a, b) (+inf if no step)
+    float lunit;      // mm of chord per unit of u_a
+    float fin, fout;  // clip inside the first / last slab (local coordinate in [0,1])
+    int i0, ns;       // first slab index along a, number of slabs
+    int ta, tb, tc;   // table offsets of axes a, b, c, pre-shifted by HALO_LO
+    int steps;        // bits 0-1: step of b (+1 -> 1, -1 -> 3, 0 -> 0); bits 2-3: same for c
 };
 
-// Register-resident pick of element i of a 3-array (avoids local-memory indexing).
 template <class T>
 __device__ __forceinline__ T sel3(const T (&v)[3], int i) {
     return i == 0 ? v[0] : (i == 1 ? v[1] : v[2]);
@@ -79,20 +89,17 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
         }
     }
     if (!(amax > amin)) return false;
-    // dominant axis in voxel units
     const double ax = fabs(D[0]), ay = fabs(D[1]), az = fabs(D[2]);
-    int a = (ax >= ay && ax >= az) ? 0 : ((ay >= az) ? 1 : 2);
-    int b = (a == 0) ? 1 : 0;
-    int c = (a == 2) ? 1 : 2;
+    const int a = (ax >= ay && ax >= az) ? 0 : ((ay >= az) ? 1 : 2);
+    const int b = (a == 0) ? 1 : 0;
+    const int c = (a == 2) ? 1 : 2;
     const double Da = sel3(D, a), u1a = sel3(u1, a);
     const double Db = sel3(D, b), Dc = sel3(D, c), u1b = sel3(u1, b), u1c = sel3(u1, c);
     double ua_in = u1a + amin * Da, ua_out = u1a + amax * Da;
     if (Da < 0.0) { double t = ua_in; ua_in = ua_out; ua_out = t; }
     const int na = sel3(g.n, a);
-    int i0 = (int)floor(ua_in);
-    int il = (int)ceil(ua_out) - 1;
-    i0 = max(i0, 0);
-    il = min(il, na - 1);
+    int i0 = max((int)floor(ua_in), 0);
+    int il = min((int)ceil(ua_out) - 1, na - 1);
     if (il < i0) return false;
     const double rDa = 1.0 / Da;
     const double sb = Db * rDa, sc = Dc * rDa;
@@ -100,19 +107,22 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     L.sc = sc;
     L.wb0 = u1b + ((double)i0 - u1a) * sb;
     L.wc0 = u1c + ((double)i0 - u1a) * sc;
-    L.isb = (sb != 0.0) ? (float)(1.0 / fabs(sb)) : CUDART_INF_F;
-    L.isc = (sc != 0.0) ? (float)(1.0 / fabs(sc)) : CUDART_INF_F;
+    // crossing inside a slab, from the fraction f of the minor position at the slab plane:
+    //   step +1: plane floor+1 at (1 - f)/|s|;  step -1: plane floor at f/|s|;  no step: never
+    const float isb = (float)(1.0 / fabs(sb)), isc = (float)(1.0 / fabs(sc));
+    L.ab = sb > 0.0 ? -isb : (sb < 0.0 ? isb : 0.0f);
+    L.bb = sb > 0.0 ? isb : (sb < 0.0 ? 0.0f : CUDART_INF_F);
+    L.ac = sc > 0.0 ? -isc : (sc < 0.0 ? isc : 0.0f);
+    L.bc = sc > 0.0 ? isc : (sc < 0.0 ? 0.0f : CUDART_INF_F);
     L.lunit = (float)(Lmm * fabs(rDa));
     L.fin = fminf(fmaxf((float)(ua_in - (double)i0), 0.0f), 1.0f);
     L.fout = fminf(fmaxf((float)(ua_out - (double)il), 0.0f), 1.0f);
     L.i0 = i0;
     L.ns = il - i0 + 1;
-    L.sa = sel3(g.stride, a);
-    L.sbs = sel3(g.stride, b);
-    L.scs = sel3(g.stride, c);
-    L.nb = sel3(g.n, b);
-    L.nc = sel3(g.n, c);
-    L.steps = (sb > 0.0 ? 1 : 0) | (sb < 0.0 ? 2 : 0) | (sc > 0.0 ? 4 : 0) | (sc < 0.0 ? 8 : 0);
+    L.ta = sel3(g.toff, a) + HALO_LO;
+    L.tb = sel3(g.toff, b) + HALO_LO;
+    L.tc = sel3(g.toff, c) + HALO_LO;
+    L.steps = (sb > 0.0 ? 1 : (sb < 0.0 ? 3 : 0)) | (sc > 0.0 ? 4 : (sc < 0.0 ? 12 : 0));
     return true;
 }
 
@@ -129,52 +139,50 @@ __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     L.wc0 = shfl_d(s.wc0, src);
     L.sb = shfl_d(s.sb, src);
     L.sc = shfl_d(s.sc, src);
-    L.isb = __shfl_sync(0xffffffffu, s.isb, src);
-    L.isc = __shfl_sync(0xffffffffu, s.isc, src);
+    L.ab = __shfl_sync(0xffffffffu, s.ab, src);
+    L.bb = __shfl_sync(0xffffffffu, s.bb, src);
+    L.ac = __shfl_sync(0xffffffffu, s.ac, src);
+    L.bc = __shfl_sync(0xffffffffu, s.bc, src);
     L.lunit = __shfl_sync(0xffffffffu, s.lunit, src);
     L.fin = __shfl_sync(0xffffffffu, s.fin, src);
     L.fout = __shfl_sync(0xffffffffu, s.fout, src);
     L.i0 = __shfl_sync(0xffffffffu, s.i0, src);
     L.ns = __shfl_sync(0xffffffffu, s.ns, src);
-    L.sa = __shfl_sync(0xffffffffu, s.sa, src);
-    L.sbs = __shfl_sync(0xffffffffu, s.sbs, src);
-    L.scs = __shfl_sync(0xffffffffu, s.scs, src);
-    L.nb = __shfl_sync(0xffffffffu, s.nb, src);
-    L.nc = __shfl_sync(0xffffffffu, s.nc, src);
+    L.ta = __shfl_sync(0xffffffffu, s.ta, src);
+    L.tb = __shfl_sync(0xffffffffu, s.tb, src);
+    L.tc = __shfl_sync(0xffffffffu, s.tc, src);
     L.steps = __shfl_sync(0xffffffffu, s.steps, src);
     return L;
 }
 
-// The (up to) three pieces of slab k of a LOR: calls emit(j, len) for each piece of
-// positive length whose voxel lies in the volume.
-template <class Emit>
-__device__ __forceinline__ void slab_pieces(const Lor& L, int k, Emit&& emit) {
+// The (up to) three pieces of slab k: j[p] = brick index, len[p] = chord length in mm
+// (0 for an empty piece). tab = shared per-axis index tables.
+__device__ __forceinline__ void slab_pieces(const Lor& L, int k, const int* __restrict__ tab, int j[3],
+                                            float len[3]) {
     const double wb = fma((double)k, L.sb, L.wb0);
     const double wc = fma((double)k, L.sc, L.wc0);
     const double fbb = floor(wb), fcc = floor(wc);
-    const int bb = (int)fbb, cc = (int)fcc;
-    const float fb = (float)(wb - fbb), fc = (float)(wc - fcc);
-    const int stb = (L.steps & 1) ? 1 : ((L.steps & 2) ? -1 : 0);
-    const int stc = (L.steps & 4) ? 1 : ((L.steps & 8) ? -1 : 0);
-    // local crossing positions in [0, inf) along u_a from the slab's lower plane
-    const float db = (stb > 0) ? (1.0f - fb) * L.isb : ((stb < 0) ? fb * L.isb : CUDART_INF_F);
-    const float dc = (stc > 0) ? (1.0f - fc) * L.isc : ((stc < 0) ? fc * L.isc : CUDART_INF_F);
+    const int ib = (int)fbb, ic = (int)fcc;
+    const float db = fmaf((float)(wb - fbb), L.ab, L.bb);
+    const float dc = fmaf((float)(wc - fcc), L.ac, L.bc);
     const float dlo = (k == 0) ? L.fin : 0.0f;
     const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;
     const float x1 = fminf(db, dc), x2 = fmaxf(db, dc);
     const float q1 = fminf(fmaxf(x1, dlo), dhi);
     const float q2 = fminf(fmaxf(x2, dlo), dhi);
-    const int ja = (L.i0 + k) * L.sa;
-    const float s[3] = {dlo, q1, q2};
-    const float e[3] = {q1, q2, dhi};
-#pragma unroll
-    for (int p = 0; p < 3; ++p) {
-        const int ib = bb + ((s[p] >= db) ? stb : 0);
-        const int ic = cc + ((s[p] >= dc) ? stc : 0);
-        const float len = (e[p] - s[p]) * L.lunit;
-        const bool ok = (e[p] > s[p]) && ((unsigned)ib < (unsigned)L.nb) && ((unsigned)ic < (unsigned)L.nc);
-        emit(ok, ja + ib * L.sbs + ic * L.scs, len);
-    }
+    // step of each minor axis: +1, -1 or 0 (bits of L.steps)
+    const int stb = ((L.steps & 3) == 1) - ((L.steps & 3) == 3);
+    const int stc = ((L.steps & 12) == 4) - ((L.steps & 12) == 12);
+    const int Ja = tab[L.ta + L.i0 + k];
+    const int Jb0 = tab[L.tb + ib], Jb1 = tab[L.tb + ib + stb];
+    const int Jc0 = tab[L.tc + ic], Jc1 = tab[L.tc + ic + stc];
+    // piece 0 before both crossings, piece 2 after both, piece 1 after the first one
+    j[0] = Ja + Jb0 + Jc0;
+    j[1] = Ja + ((db <= dc) ? (Jb1 + Jc0) : (Jb0 + Jc1));
+    j[2] = Ja + Jb1 + Jc1;
+    len[0] = (q1 - dlo) * L.lunit;
+    len[1] = (q2 - q1) * L.lunit;
+    len[2] = (dhi - q2) * L.lunit;
 }
 
 __device__ __forceinline__ float warp_sum(float v) {
@@ -183,22 +191,33 @@ __device__ __forceinline__ float warp_sum(float v) {
     return v;
 }
 
-// Loads event idx (6 floats) of an AoS array: three 8-byte loads (24-byte records are
-// 8-byte aligned); consecutive lanes read consecutive records (coalesced 768 B / warp).
+// Loads event idx (6 floats): three 8-byte streaming loads; consecutive lanes read
+// consecutive 24-byte records (768 contiguous bytes per warp).
 __device__ __forceinline__ void load_event(const float* __restrict__ events, int64_t idx, float ev[6]) {
     const float2* p = reinterpret_cast<const float2*>(events + 6 * idx);
     float2 a = __ldcs(p), b = __ldcs(p + 1), c = __ldcs(p + 2);
     ev[0] = a.x; ev[1] = a.y; ev[2] = b.x; ev[3] = b.y; ev[4] = c.x; ev[5] = c.y;
 }
 
-// MODE 0: fused forward + back-projection into c (step 1).
+// Dynamic shared memory: int tab[tsize] (rounded to 8 B), then per warp `cap` path
+// pieces of (int j, float len) packed as int2.
+// MODE 0: fused forward + back-projection into cb (step 1).
 // MODE 1: forward projection only, fp written to fp_out[i] (tests).
 template <int MODE>
-__global__ void __launch_bounds__(256) k_project(const float* __restrict__ events, int64_t n,
-                                                 const float* __restrict__ f, float* __restrict__ c,
-                                                 float* __restrict__ fp_out, GridGeom g) {
+__global__ void __launch_bounds__(256, 3) k_project(const float* __restrict__ events, int64_t n,
+                                                    const float* __restrict__ fb, float* __restrict__ cb,
+                                                    float* __restrict__ fp_out, const int* __restrict__ tab_g,
+                                                    GridGeom g, int cap) {
+    extern __shared__ __align__(16) int smem[];
+    int* tab = smem;
+    const int tpad = (g.tsize + 1) & ~1;
+    for (int t = threadIdx.x; t < g.tsize; t += blockDim.x) tab[t] = tab_g[t];
+    __syncthreads();
     const int lane = threadIdx.x & 31;
-    const int64_t warp = (int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5);
+    const int wib = threadIdx.x >> 5;
+    int2* path = reinterpret_cast<int2*>(smem + tpad) + (size_t)wib * cap;
+    const unsigned lt = (1u << lane) - 1u;
+    const int64_t warp = (int64_t)blockIdx.x * (blockDim.x >> 5) + wib;
     const int64_t nwarps = (int64_t)gridDim.x * (blockDim.x >> 5);
     for (int64_t base = warp * 32; base < n; base += nwarps * 32) {
         const int64_t idx = base + lane;
@@ -215,54 +234,140 @@ __global__ void __launch_bounds__(256) k_project(const float* __restrict__ event
             const int src = __ffs(mask) - 1;
             mask &= mask - 1;
             const Lor L = shfl_lor(mine, src);
+            // pass 1: geometry -> compacted path pieces in shared memory
+            int cnt = 0;
+            for (int k0 = 0; k0 < L.ns; k0 += 32) {
+                const int k = k0 + lane;
+                int j[3];
+                float len[3];
+                bool v[3] = {false, false, false};
+                if (k < L.ns) {
+                    slab_pieces(L, k, tab, j, len);
+#pragma unroll
+                    for (int p = 0; p < 3; ++p) v[p] = len[p] > 0.0f;
+                }
+#pragma unroll
+                for (int p = 0; p < 3; ++p) {
+                    const unsigned bal = __ballot_sync(0xffffffffu, v[p]);
+                    if (v[p]) path[cnt + __popc(bal & lt)] = make_int2(j[p], __float_as_int(len[p]));
+                    cnt += __popc(bal);
+                }
+            }
+            __syncwarp();
+            // pass 2: forward projection, lane m <- piece m
             float acc = 0.0f;
-            for (int k = lane; k < L.ns; k += 32) {
-                slab_pieces(L, k, [&](bool v, int j, float len) {
-                    if (v) acc = fmaf(__ldg(f + j), len, acc);
-                });
+            for (int m = lane; m < cnt; m += 32) {
+                const int2 q = path[m];
+                acc = fmaf(__ldg(fb + q.x), __int_as_float(q.y), acc);
             }
             const float fp = warp_sum(acc);
             if (MODE == 1) {
                 if (lane == 0) fp_out[base + src] = fp;
-                continue;
+            } else if (fp > 0.0f) {  // reading S7: skip events with fp <= 0
+                // pass 3: back-projection
+                const float inv = 1.0f / fp;
+                for (int m = lane; m < cnt; m += 32) {
+                    const int2 q = path[m];
+                    atomicAdd(cb + q.x, __int_as_float(q.y) * inv);
+                }
             }
-            if (!(fp > 0.0f)) continue;  // reading S7: skip events with fp <= 0
-            const float inv = 1.0f / fp;
-            for (int k = lane; k < L.ns; k += 32) {
-                slab_pieces(L, k, [&](bool v, int j, float len) {
-                    if (v) atomicAdd(c + j, len * inv);
-                });
-            }
+            __syncwarp();
         }
     }
 }
 
-// Step 2: f_j <- f_j * c_j / s_j where c_j > 0 and s_j > 0; c_j <- 0 (next subset).
+// ---------------------------------------------------------------- brick <-> row layouts
+// One thread per brick (8 voxels). Brick b = bx + BX*(by + BY*bz) holds padded voxels
+// (2bx+dx, 2by+dy, 2bz+dz) at 8b + dx + 2dy + 4dz; real voxel i = p - HALO_LO.
+struct BrickIt {
+    int BX, BY, BZ;
+    int64_t nb;
+};
+
+__device__ __forceinline__ bool real_voxel(const GridGeom& g, int px, int py, int pz, int64_t& r) {
+    const int ix = px - HALO_LO, iy = py - HALO_LO, iz = pz - HALO_LO;
+    if ((unsigned)ix >= (unsigned)g.n[0] || (unsigned)iy >= (unsigned)g.n[1] || (unsigned)iz >= (unsigned)g.n[2])
+        return false;
+    r = (int64_t)ix + (int64_t)g.n[0] * ((int64_t)iy + (int64_t)g.n[1] * iz);
+    return true;
+}
+
+// row (x-fastest, caller) -> bricks (halo = 0)
+__global__ void __launch_bounds__(256) k_row_to_brick(const float* __restrict__ row, float* __restrict__ br,
+                                                      GridGeom g, BrickIt it) {
+    for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
+        const int bx = (int)(b % it.BX);
+        const int64_t t = b / it.BX;
+        const int by = (int)(t % it.BY), bz = (int)(t / it.BY);
+        float v[8];
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+            int64_t r;
+            v[q] = real_voxel(g, 2 * bx + (q & 1), 2 * by + ((q >> 1) & 1), 2 * bz + (q >> 2), r) ? __ldg(row + r) : 0.0f;
+        }
+        float4* o = reinterpret_cast<float4*>(br + 8 * b);
+        o[0] = make_float4(v[0], v[1], v[2], v[3]);
+        o[1] = make_float4(v[4], v[5], v[6], v[7]);
+    }
+}
+
+// bricks -> row (real voxels only); optionally zeroes the bricks afterwards
+__global__ void __launch_bounds__(256) k_brick_to_row(float* __restrict__ br, float* __restrict__ row, GridGeom g,
+                                                      BrickIt it, int zero) {
+    for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
+        const int bx = (int)(b % it.BX);
+        const int64_t t = b / it.BX;
+        const int by = (int)(t % it.BY), bz = (int)(t / it.BY);
+        float4* p = reinterpret_cast<float4*>(br + 8 * b);
+        const float4 a = p[0], c = p[1];
+        const float v[8] = {a.x, a.y, a.z, a.w, c.x, c.y, c.z, c.w};
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+            int64_t r;
+            if (real_voxel(g, 2 * bx + (q & 1), 2 * by + ((q >> 1) & 1), 2 * bz + (q >> 2), r)) row[r] = v[q];
+        }
+        if (zero) {
+            p[0] = make_float4(0.f, 0.f, 0.f, 0.f);
+            p[1] = make_float4(0.f, 0.f, 0.f, 0.f);
+        }
+    }
+}
+
+// Step 2: f_j <- f_j * c_j / s_j where c_j > 0 and s_j > 0 (reading S9), c_j <- 0.
+// Updates the brick copy fb and writes the caller's row-layout f. Halo voxels keep
+// fb = 0 (sb = 0 there, so the guard leaves them unchanged).
 __device__ __forceinline__ float upd1(float f, float c, float s) {
     return (c > 0.0f && s > 0.0f) ? f * __fdiv_rn(c, s) : f;
 }
 
-// vec = 1 when f, c and s are 16-byte aligned (float4 path), else scalar throughout.
-__global__ void __launch_bounds__(256) k_update(float* __restrict__ f, float* __restrict__ c,
-                                                const float* __restrict__ s, int64_t V, int vec) {
-    const int64_t n4 = vec ? (V >> 2) : 0;
-    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
-    float4* f4 = reinterpret_cast<float4*>(f);
-    float4* c4 = reinterpret_cast<float4*>(c);
-    const float4* s4 = reinterpret_cast<const float4*>(s);
-    const float4 z = make_float4(0.f, 0.f, 0.f, 0.f);
-    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n4; i += stride) {
-        float4 fv = f4[i], cv = __ldcs(c4 + i), sv = __ldg(s4 + i);
-        fv.x = upd1(fv.x, cv.x, sv.x);
-        fv.y = upd1(fv.y, cv.y, sv.y);
-        fv.z = upd1(fv.z, cv.z, sv.z);
-        fv.w = upd1(fv.w, cv.w, sv.w);
-        f4[i] = fv;
-        c4[i] = z;
-    }
-    for (int64_t i = (n4 << 2) + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < V; i += stride) {
-        f[i] = upd1(f[i], c[i], s[i]);
-        c[i] = 0.0f;
+__global__ void __launch_bounds__(256) k_update(float* __restrict__ fb, float* __restrict__ cb,
+                                                const float* __restrict__ sb, float* __restrict__ f_row, GridGeom g,
+                                                BrickIt it) {
+    for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
+        float4* F = reinterpret_cast<float4*>(fb + 8 * b);
+        float4* C = reinterpret_cast<float4*>(cb + 8 * b);
+        const float4* S = reinterpret_cast<const float4*>(sb + 8 * b);
+        float4 f0 = F[0], f1 = F[1];
+        const float4 c0 = __ldcs(C), c1 = __ldcs(C + 1), s0 = __ldg(S), s1 = __ldg(S + 1);
+        f0.x = upd1(f0.x, c0.x, s0.x); f0.y = upd1(f0.y, c0.y, s0.y);
+        f0.z = upd1(f0.z, c0.z, s0.z); f0.w = upd1(f0.w, c0.w, s0.w);
+        f1.x = upd1(f1.x, c1.x, s1.x); f1.y = upd1(f1.y, c1.y, s1.y);
+        f1.z = upd1(f1.z, c1.z, s1.z); f1.w = upd1(f1.w, c1.w, s1.w);
+        F[0] = f0;
+        F[1] = f1;
+        C[0] = make_float4(0.f, 0.f, 0.f, 0.f);
+        C[1] = make_float4(0.f, 0.f, 0.f, 0.f);
+        if (f_row) {
+            const int bx = (int)(b % it.BX);
+            const int64_t t = b / it.BX;
+            const int by = (int)(t % it.BY), bz = (int)(t / it.BY);
+            const float v[8] = {f0.x, f0.y, f0.z, f0.w, f1.x, f1.y, f1.z, f1.w};
+#pragma unroll
+            for (int q = 0; q < 8; ++q) {
+                int64_t r;
+                if (real_voxel(g, 2 * bx + (q & 1), 2 * by + ((q >> 1) & 1), 2 * bz + (q >> 2), r)) f_row[r] = v[q];
+            }
+        }
     }
 }
 

@@ -40,7 +40,7 @@ class Dist(ctypes.Structure):
 
 class Stats(ctypes.Structure):
     _fields_ = [("launches", ctypes.c_int64), ("subsets", ctypes.c_int64), ("events", ctypes.c_int64),
-                ("timed_subsets", ctypes.c_int64), ("project_ms", ctypes.c_double),
+                ("timed_subsets", ctypes.c_int64), ("convert_ms", ctypes.c_double), ("project_ms", ctypes.c_double),
                 ("combine_ms", ctypes.c_double), ("update_ms", ctypes.c_double), ("h2d_ms", ctypes.c_double)]
 
     def as_dict(self) -> dict:

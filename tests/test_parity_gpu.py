@@ -198,7 +198,8 @@ def test_c1_full_reconstruction(pkg, iters):
     assert rel_l2(got, ref) <= REL_L2_RECON
     assert np.all(got > 0)
     st = rec.stats()
-    assert st["subsets"] == iters * cfg.n_subsets and st["launches"] == 2 * iters * cfg.n_subsets
+    # one f -> brick conversion, then (project, update) per subset
+    assert st["subsets"] == iters * cfg.n_subsets and st["launches"] == 2 * iters * cfg.n_subsets + 1
     rec.close()
 
 
