@@ -51,13 +51,17 @@ def build_l2peak() -> str:
     return L2PEAK_SO
 
 
-def build(force: bool = False, verbose: bool = False) -> str:
-    if not force and not needs_build():
+def build(force: bool = False, verbose: bool = False, defines=(), out: str | None = None) -> str:
+    """Builds liblmosem.so (and libl2peak.so). `defines`/`out` build an A/B variant of
+    the kernels (e.g. defines=["LMK_TRASH=0"], out=".../liblmosem_v.so")."""
+    if out is None and not force and not needs_build():
         return SO
-    build_l2peak()
+    target = out or SO
+    if out is None:
+        build_l2peak()
     inc, lib = nccl_paths()
-    tmp = SO + f".tmp{os.getpid()}"
-    cmd = [NVCC, *ARCH, "-O3", "-std=c++17", "-lineinfo", "-Xptxas", "-v",
+    tmp = target + f".tmp{os.getpid()}"
+    cmd = [NVCC, *ARCH, "-O3", "-std=c++17", "-lineinfo", "-Xptxas", "-v", *[f"-D{d}" for d in defines],
            "-Xcompiler", "-fPIC,-fvisibility=hidden", "-shared",
            "-I", os.path.join(ROOT, "include"), "-I", CSRC, "-I", inc,
            os.path.join(CSRC, "lmosem.cu"), "-o", tmp,
@@ -65,12 +69,13 @@ def build(force: bool = False, verbose: bool = False) -> str:
     res = subprocess.run(cmd, capture_output=True, text=True)
     if res.returncode != 0:
         raise RuntimeError("nvcc failed:\n" + res.stdout + res.stderr)
-    with open(os.path.join(PKG, "build_ptxas.log"), "w") as fh:
-        fh.write(" ".join(cmd) + "\n" + res.stdout + res.stderr)
+    if out is None:
+        with open(os.path.join(PKG, "build_ptxas.log"), "w") as fh:
+            fh.write(" ".join(cmd) + "\n" + res.stdout + res.stderr)
     if verbose:
         print(res.stderr)
-    os.replace(tmp, SO)
-    return SO
+    os.replace(tmp, target)
+    return target
 
 
 if __name__ == "__main__":

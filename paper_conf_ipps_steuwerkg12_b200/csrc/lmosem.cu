@@ -118,15 +118,16 @@ lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
 lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* fp_out, int mode) {
     if (n <= 0) return LMOSEM_OK;
     const int64_t warps_needed = (n + 31) / 32;
-    const int64_t blocks_needed = (warps_needed + 7) / 8;
+    const int64_t wpb = lmk::PROJ_THREADS / 32;
+    const int64_t blocks_needed = (warps_needed + wpb - 1) / wpb;
     const int64_t cap = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm;
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
     const float* evf = reinterpret_cast<const float*>(ev);
     if (mode == 0)
-        lmk::k_project<0><<<grid, 256, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, ctx->c, nullptr, ctx->tab,
+        lmk::k_project<0><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, ctx->c, nullptr, ctx->tab,
                                                                       ctx->geom, ctx->cap);
     else
-        lmk::k_project<1><<<grid, 256, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, nullptr, fp_out, ctx->tab,
+        lmk::k_project<1><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, nullptr, fp_out, ctx->tab,
                                                                       ctx->geom, ctx->cap);
     CK(cudaGetLastError());
     ctx->st.launches++;
@@ -294,8 +295,10 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         for (int k = 0; k < 3; ++k)
             for (int p = 0; p < ctx->geom.P[k]; ++p) tab[ctx->geom.toff[k] + p] = (int)(M[k] * (p >> 1) + m[k] * (p & 1));
     }
-    ctx->cap = 3 * std::max(dims[0], std::max(dims[1], dims[2])) + 8;
-    ctx->proj_smem = sizeof(int) * (size_t)((ctx->geom.tsize + 1) & ~1) + 8 * sizeof(int2) * (size_t)ctx->cap;
+    // <= 3 pieces per dominant-axis slab, + the trash slot
+    ctx->cap = 3 * std::max(dims[0], std::max(dims[1], dims[2])) + 1;
+    ctx->proj_smem = sizeof(int) * (size_t)((ctx->geom.tsize + 1) & ~1) +
+                     (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
 
     lmosem_status s = LMOSEM_OK;
     auto cuda = [&](cudaError_t e, const char* what) {
@@ -317,7 +320,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
          "smem attr");
     cuda(cudaFuncSetAttribute(lmk::k_project<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
          "smem attr");
-    cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, 256,
+    cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, lmk::PROJ_THREADS,
                                                        ctx->proj_smem),
          "occupancy");
     if (ctx->proj_blocks_per_sm < 1) ctx->proj_blocks_per_sm = 1;

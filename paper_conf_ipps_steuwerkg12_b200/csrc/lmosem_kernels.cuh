@@ -5,13 +5,13 @@
 //   - setup, per LOR in float64 (one lane per event of a 32-event batch, broadcast by
 //     shuffles): clip to the volume, dominant axis a (largest |du_a| in voxel units),
 //     minor-axis positions at the first slab plane and slopes du_b/du_a, du_c/du_a
-//     (|slope| <= 1);
+//     (|slope| <= 1), the positions kept in Q24.40 fixed point;
 //   - pass 1 (geometry): lane k takes slabs k, k+32, ... of the dominant axis. Each minor
 //     axis crosses at most one plane inside a slab, so a slab holds <= 3 pieces; the
-//     minor positions at the slab plane are one float64 FMA and the crossings are float32
-//     relative to that plane (values in [0,1], ~1e-7 voxel absolute error wherever the
-//     slab lies). The pieces (j, len) are compacted into the warp's shared-memory path
-//     buffer, slab-major;
+//     minor positions at the slab plane are one 64-bit integer multiply-add and the
+//     crossings are float32 relative to that plane (values in [0,1], ~1e-7 voxel absolute
+//     error wherever the slab lies). The pieces (j, len) are compacted into the warp's
+//     shared-memory path buffer, slab-major;
 //   - pass 2 (forward projection, lines 9-10): lane m reads piece m and gathers f — lanes
 //     hold consecutive pieces of one path, so they share 32-byte sectors of the brick
 //     layout below; warp reduction gives fp;
@@ -42,11 +42,16 @@ struct GridGeom {
     double inv_v[3];  // 1 / voxel size (1/mm)
 };
 
+// Minor-axis positions are fixed point Q24.40 (int64, 2^-40 voxel): exact integer
+// stepping w(k) = w0 + k*s, floor = w >> 40, fraction = low 40 bits. The slope error
+// (<= 2^-41 per slab) accumulates to < 1e-9 voxel over 600 slabs.
+constexpr int FIX_BITS = 40;
+
 // Per-LOR traversal state (broadcast lane -> warp by shuffles).
 struct Lor {
-    double wb0, wc0;  // minor-axis positions (voxel units) at the plane u_a = i0
-    double sb, sc;    // du_b/du_a, du_c/du_a
-    float ab, bb, ac, bc;  // crossing position in a slab: d = fma(frac, a, b) (+inf if no step)
+    long long wb0, wc0;  // minor-axis positions at the plane u_a = i0 (Q24.40 voxels)
+    long long sb, sc;    // du_b/du_a, du_c/du_a (Q24.40)
+    float ab, bb, ac, bc;  // crossing offset in a slab: d = fma(g, a, b) (+inf if no step)
     float lunit;      // mm of chord per unit of u_a
     float fin, fout;  // clip inside the first / last slab (local coordinate in [0,1])
     int i0, ns;       // first slab index along a, number of slabs
@@ -103,17 +108,18 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     if (il < i0) return false;
     const double rDa = 1.0 / Da;
     const double sb = Db * rDa, sc = Dc * rDa;
-    L.sb = sb;
-    L.sc = sc;
-    L.wb0 = u1b + ((double)i0 - u1a) * sb;
-    L.wc0 = u1c + ((double)i0 - u1a) * sc;
-    // crossing inside a slab, from the fraction f of the minor position at the slab plane:
-    //   step +1: plane floor+1 at (1 - f)/|s|;  step -1: plane floor at f/|s|;  no step: never
-    const float isb = (float)(1.0 / fabs(sb)), isc = (float)(1.0 / fabs(sc));
-    L.ab = sb > 0.0 ? -isb : (sb < 0.0 ? isb : 0.0f);
-    L.bb = sb > 0.0 ? isb : (sb < 0.0 ? 0.0f : CUDART_INF_F);
-    L.ac = sc > 0.0 ? -isc : (sc < 0.0 ? isc : 0.0f);
-    L.bc = sc > 0.0 ? isc : (sc < 0.0 ? 0.0f : CUDART_INF_F);
+    const double fx = (double)(1LL << FIX_BITS);
+    L.sb = __double2ll_rn(sb * fx);
+    L.sc = __double2ll_rn(sc * fx);
+    L.wb0 = __double2ll_rn((u1b + ((double)i0 - u1a) * sb) * fx);
+    L.wc0 = __double2ll_rn((u1c + ((double)i0 - u1a) * sc) * fx);
+    // crossing inside a slab: distance g (Q.40 units) to the next plane in the direction
+    // of travel, divided by |slope|: d = g * 2^-40 / |s| (no step: never, d = +inf)
+    const float isb = (float)(1.0 / (fabs(sb) * fx)), isc = (float)(1.0 / (fabs(sc) * fx));
+    L.ab = sb != 0.0 ? isb : 0.0f;
+    L.bb = sb != 0.0 ? 0.0f : CUDART_INF_F;
+    L.ac = sc != 0.0 ? isc : 0.0f;
+    L.bc = sc != 0.0 ? 0.0f : CUDART_INF_F;
     L.lunit = (float)(Lmm * fabs(rDa));
     L.fin = fminf(fmaxf((float)(ua_in - (double)i0), 0.0f), 1.0f);
     L.fout = fminf(fmaxf((float)(ua_out - (double)il), 0.0f), 1.0f);
@@ -133,12 +139,29 @@ __device__ __forceinline__ double shfl_d(double v, int src) {
     return __hiloint2double(hi, lo);
 }
 
+__device__ __forceinline__ long long shfl_ll(long long v, int src) {
+    int lo = (int)(unsigned long long)v, hi = (int)((unsigned long long)v >> 32);
+    lo = __shfl_sync(0xffffffffu, lo, src);
+    hi = __shfl_sync(0xffffffffu, hi, src);
+    return (long long)(((unsigned long long)(unsigned)hi << 32) | (unsigned)lo);
+}
+
+// Q24.40 position w -> floor (int) and the exact distance to the next voxel plane in
+// the direction of travel (up: 2^40 - frac, down: frac), converted to float with full
+// relative precision (the crossing offset divides it by |slope|, so an absolute
+// rounding error here would be amplified for shallow minor axes).
+__device__ __forceinline__ float fix_to_plane(long long w, bool up, int& fl) {
+    fl = (int)(w >> FIX_BITS);
+    const unsigned long long frac = (unsigned long long)w & ((1ULL << FIX_BITS) - 1ULL);
+    return __ull2float_rn(up ? (1ULL << FIX_BITS) - frac : frac);
+}
+
 __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     Lor L;
-    L.wb0 = shfl_d(s.wb0, src);
-    L.wc0 = shfl_d(s.wc0, src);
-    L.sb = shfl_d(s.sb, src);
-    L.sc = shfl_d(s.sc, src);
+    L.wb0 = shfl_ll(s.wb0, src);
+    L.wc0 = shfl_ll(s.wc0, src);
+    L.sb = shfl_ll(s.sb, src);
+    L.sc = shfl_ll(s.sc, src);
     L.ab = __shfl_sync(0xffffffffu, s.ab, src);
     L.bb = __shfl_sync(0xffffffffu, s.bb, src);
     L.ac = __shfl_sync(0xffffffffu, s.ac, src);
@@ -155,34 +178,35 @@ __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     return L;
 }
 
-// The (up to) three pieces of slab k: j[p] = brick index, len[p] = chord length in mm
-// (0 for an empty piece). tab = shared per-axis index tables.
-__device__ __forceinline__ void slab_pieces(const Lor& L, int k, const int* __restrict__ tab, int j[3],
-                                            float len[3]) {
-    const double wb = fma((double)k, L.sb, L.wb0);
-    const double wc = fma((double)k, L.sc, L.wc0);
-    const double fbb = floor(wb), fcc = floor(wc);
-    const int ib = (int)fbb, ic = (int)fcc;
-    const float db = fmaf((float)(wb - fbb), L.ab, L.bb);
-    const float dc = fmaf((float)(wc - fcc), L.ac, L.bc);
+// The (up to) three pieces of slab k: j = brick index, l = chord length in mm (0 for
+// an empty piece). tab = per-axis brick index tables (shared memory, 2-5 KB).
+struct Pieces {
+    int j0, j1, j2;
+    float l0, l1, l2;
+};
+
+__device__ __forceinline__ Pieces slab_pieces(const Lor& L, int k, int stb, int stc, const int* __restrict__ tab) {
+    int ib, ic;
+    const float gb = fix_to_plane(L.wb0 + (long long)k * L.sb, stb > 0, ib);
+    const float gc = fix_to_plane(L.wc0 + (long long)k * L.sc, stc > 0, ic);
+    const float db = fmaf(gb, L.ab, L.bb);  // crossing offsets along u_a in the slab
+    const float dc = fmaf(gc, L.ac, L.bc);
     const float dlo = (k == 0) ? L.fin : 0.0f;
     const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;
-    const float x1 = fminf(db, dc), x2 = fmaxf(db, dc);
-    const float q1 = fminf(fmaxf(x1, dlo), dhi);
-    const float q2 = fminf(fmaxf(x2, dlo), dhi);
-    // step of each minor axis: +1, -1 or 0 (bits of L.steps)
-    const int stb = ((L.steps & 3) == 1) - ((L.steps & 3) == 3);
-    const int stc = ((L.steps & 12) == 4) - ((L.steps & 12) == 12);
+    const float q1 = fminf(fmaxf(fminf(db, dc), dlo), dhi);
+    const float q2 = fminf(fmaxf(fmaxf(db, dc), dlo), dhi);
     const int Ja = tab[L.ta + L.i0 + k];
     const int Jb0 = tab[L.tb + ib], Jb1 = tab[L.tb + ib + stb];
     const int Jc0 = tab[L.tc + ic], Jc1 = tab[L.tc + ic + stc];
     // piece 0 before both crossings, piece 2 after both, piece 1 after the first one
-    j[0] = Ja + Jb0 + Jc0;
-    j[1] = Ja + ((db <= dc) ? (Jb1 + Jc0) : (Jb0 + Jc1));
-    j[2] = Ja + Jb1 + Jc1;
-    len[0] = (q1 - dlo) * L.lunit;
-    len[1] = (q2 - q1) * L.lunit;
-    len[2] = (dhi - q2) * L.lunit;
+    Pieces P;
+    P.j0 = Ja + Jb0 + Jc0;
+    P.j1 = Ja + ((db <= dc) ? (Jb1 + Jc0) : (Jb0 + Jc1));
+    P.j2 = Ja + Jb1 + Jc1;
+    P.l0 = (q1 - dlo) * L.lunit;
+    P.l1 = (q2 - q1) * L.lunit;
+    P.l2 = (dhi - q2) * L.lunit;
+    return P;
 }
 
 __device__ __forceinline__ float warp_sum(float v) {
@@ -199,15 +223,42 @@ __device__ __forceinline__ void load_event(const float* __restrict__ events, int
     ev[0] = a.x; ev[1] = a.y; ev[2] = b.x; ev[3] = b.y; ev[4] = c.x; ev[5] = c.y;
 }
 
-// Dynamic shared memory: int tab[tsize] (rounded to 8 B), then per warp `cap` path
-// pieces of (int j, float len) packed as int2.
+// Appends piece (j, l) to the warp's path buffer if v (ballot compaction, slab-major);
+// lanes without a piece store to the warp's trash slot, so the store is unconditional.
+__device__ __forceinline__ void append(int2* __restrict__ path, int trash, int& cnt, unsigned lt, bool v, int j,
+                                       float l) {
+    const unsigned bal = __ballot_sync(0xffffffffu, v);
+#if LMK_TRASH
+    path[v ? cnt + __popc(bal & lt) : trash] = make_int2(j, __float_as_int(l));
+#else
+    if (v) path[cnt + __popc(bal & lt)] = make_int2(j, __float_as_int(l));
+#endif
+    cnt += __popc(bal);
+}
+
+#ifndef LMK_CTA_THREADS
+#define LMK_CTA_THREADS 256  // 8 warps
+#endif
+#ifndef LMK_MIN_BLOCKS
+#define LMK_MIN_BLOCKS 3     // CTAs per SM
+#endif
+#ifndef LMK_TRASH
+#define LMK_TRASH 0          // 1: unconditional store to a trash slot; 0: predicated store
+#endif
+#ifndef LMK_FUSED_GATHER
+#define LMK_FUSED_GATHER 1   // 1: gather f during the geometry pass (no separate pass 2)
+#endif
+constexpr int PROJ_THREADS = LMK_CTA_THREADS;
+
+// Dynamic shared memory: int tab[tsize] (rounded up to 8 B), then per warp `cap` path
+// pieces (int j, float len) packed as int2; the last one is the warp's trash slot.
 // MODE 0: fused forward + back-projection into cb (step 1).
 // MODE 1: forward projection only, fp written to fp_out[i] (tests).
 template <int MODE>
-__global__ void __launch_bounds__(256, 3) k_project(const float* __restrict__ events, int64_t n,
-                                                    const float* __restrict__ fb, float* __restrict__ cb,
-                                                    float* __restrict__ fp_out, const int* __restrict__ tab_g,
-                                                    GridGeom g, int cap) {
+__global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const float* __restrict__ events, int64_t n,
+                                                             const float* __restrict__ fb, float* __restrict__ cb,
+                                                             float* __restrict__ fp_out, const int* __restrict__ tab_g,
+                                                             GridGeom g, int cap) {
     extern __shared__ __align__(16) int smem[];
     int* tab = smem;
     const int tpad = (g.tsize + 1) & ~1;
@@ -216,6 +267,7 @@ __global__ void __launch_bounds__(256, 3) k_project(const float* __restrict__ ev
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
     int2* path = reinterpret_cast<int2*>(smem + tpad) + (size_t)wib * cap;
+    const int trash = cap - 1;
     const unsigned lt = (1u << lane) - 1u;
     const int64_t warp = (int64_t)blockIdx.x * (blockDim.x >> 5) + wib;
     const int64_t nwarps = (int64_t)gridDim.x * (blockDim.x >> 5);
@@ -234,38 +286,58 @@ __global__ void __launch_bounds__(256, 3) k_project(const float* __restrict__ ev
             const int src = __ffs(mask) - 1;
             mask &= mask - 1;
             const Lor L = shfl_lor(mine, src);
-            // pass 1: geometry -> compacted path pieces in shared memory
+            const int stb = ((L.steps & 3) == 1) - ((L.steps & 3) == 3);
+            const int stc = ((L.steps & 12) == 4) - ((L.steps & 12) == 12);
+            // pass 1: geometry -> compacted path pieces in shared memory (uniform loop:
+            // lanes past the last slab recompute it and drop their pieces)
             int cnt = 0;
+            float acc = 0.0f;
+#if LMK_FUSED_GATHER
+            // gathers issued with the geometry; each iteration consumes the previous
+            // iteration's loads, so their latency overlaps the next slab batch
+            float g0 = 0.f, g1 = 0.f, g2 = 0.f, w0 = 0.f, w1 = 0.f, w2 = 0.f;
             for (int k0 = 0; k0 < L.ns; k0 += 32) {
-                const int k = k0 + lane;
-                int j[3];
-                float len[3];
-                bool v[3] = {false, false, false};
-                if (k < L.ns) {
-                    slab_pieces(L, k, tab, j, len);
-#pragma unroll
-                    for (int p = 0; p < 3; ++p) v[p] = len[p] > 0.0f;
-                }
-#pragma unroll
-                for (int p = 0; p < 3; ++p) {
-                    const unsigned bal = __ballot_sync(0xffffffffu, v[p]);
-                    if (v[p]) path[cnt + __popc(bal & lt)] = make_int2(j[p], __float_as_int(len[p]));
-                    cnt += __popc(bal);
-                }
+                const bool in = k0 + lane < L.ns;
+                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc, tab);
+                const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
+                append(path, trash, cnt, lt, v0, P.j0, P.l0);
+                append(path, trash, cnt, lt, v1, P.j1, P.l1);
+                append(path, trash, cnt, lt, v2, P.j2, P.l2);
+                acc = fmaf(g0, w0, acc);
+                acc = fmaf(g1, w1, acc);
+                acc = fmaf(g2, w2, acc);
+                g0 = v0 ? __ldg(fb + P.j0) : 0.f;
+                g1 = v1 ? __ldg(fb + P.j1) : 0.f;
+                g2 = v2 ? __ldg(fb + P.j2) : 0.f;
+                w0 = P.l0; w1 = P.l1; w2 = P.l2;
+            }
+            acc = fmaf(g0, w0, acc);
+            acc = fmaf(g1, w1, acc);
+            acc = fmaf(g2, w2, acc);
+            __syncwarp();
+#else
+            for (int k0 = 0; k0 < L.ns; k0 += 32) {
+                const bool in = k0 + lane < L.ns;
+                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc, tab);
+                append(path, trash, cnt, lt, in && P.l0 > 0.0f, P.j0, P.l0);
+                append(path, trash, cnt, lt, in && P.l1 > 0.0f, P.j1, P.l1);
+                append(path, trash, cnt, lt, in && P.l2 > 0.0f, P.j2, P.l2);
             }
             __syncwarp();
             // pass 2: forward projection, lane m <- piece m
-            float acc = 0.0f;
+#pragma unroll 8
             for (int m = lane; m < cnt; m += 32) {
                 const int2 q = path[m];
                 acc = fmaf(__ldg(fb + q.x), __int_as_float(q.y), acc);
             }
+#endif
             const float fp = warp_sum(acc);
             if (MODE == 1) {
                 if (lane == 0) fp_out[base + src] = fp;
             } else if (fp > 0.0f) {  // reading S7: skip events with fp <= 0
                 // pass 3: back-projection
                 const float inv = 1.0f / fp;
+#pragma unroll 8
                 for (int m = lane; m < cnt; m += 32) {
                     const int2 q = path[m];
                     atomicAdd(cb + q.x, __int_as_float(q.y) * inv);

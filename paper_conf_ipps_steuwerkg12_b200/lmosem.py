@@ -13,7 +13,8 @@ import os
 import numpy as np
 
 _PKG = os.path.dirname(os.path.abspath(__file__))
-SO_PATH = os.path.join(_PKG, "liblmosem.so")
+# LMOSEM_LIB selects an in-tree A/B build of the same library (tools/ab_variants.py)
+SO_PATH = os.environ.get("LMOSEM_LIB") or os.path.join(_PKG, "liblmosem.so")
 
 OK, EINVAL, ENOMEM, ECUDA, ENCCL, ESTATE = range(6)
 _NAMES = {0: "OK", 1: "EINVAL", 2: "ENOMEM", 3: "ECUDA", 4: "ENCCL", 5: "ESTATE"}

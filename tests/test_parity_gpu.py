@@ -34,11 +34,15 @@ def dev(a):
 
 def maxrel(got, ref):
     m = ref > 1e-3 * ref.max()
-    return float(np.max(np.abs(got[m] - ref[m]) / ref[m]))
+    v = float(np.max(np.abs(got[m] - ref[m]) / ref[m]))
+    print(f"[parity] max rel err {v:.3e} over {int(m.sum())} voxels")
+    return v
 
 
 def rel_l2(got, ref):
-    return float(np.linalg.norm(got - ref) / np.linalg.norm(ref))
+    v = float(np.linalg.norm(got - ref) / np.linalg.norm(ref))
+    print(f"[parity] rel L2 err {v:.3e}")
+    return v
 
 
 _cache = {}

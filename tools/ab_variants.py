@@ -1,0 +1,49 @@
+#!/usr/bin/env python
+"""A/B kernel variants: `build` compiles each variant (here, CPU) into variants/;
+`run` benchmarks each on the GPU (LMOSEM_LIB=<variant> python bench.py ...)."""
+import json
+import os
+import subprocess
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+VARIANTS = {
+    "default": [],
+    "unfused": ["LMK_FUSED_GATHER=0"],
+}
+
+
+def build(names):
+    from paper_conf_ipps_steuwerkg12_b200 import build as b
+    for n in names:
+        out = os.path.join(ROOT, "variants", f"liblmosem_{n}.so")
+        b.build(defines=VARIANTS[n], out=out)
+        print("built", out)
+
+
+def run(names, extra):
+    res = {}
+    for n in names:
+        env = dict(os.environ, LMOSEM_LIB=os.path.join(ROOT, "variants", f"liblmosem_{n}.so"))
+        out = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--no-cpu-baseline", "--no-e2e",
+                              "--steps", "40", "--warmup", "5", *extra], env=env, capture_output=True, text=True)
+        try:
+            d = json.loads(out.stdout.strip().splitlines()[-1])
+            res[n] = {"events_per_s": d["value"], "project_ms": d["phase_ms_per_step"]["project"]}
+        except Exception as e:  # noqa: BLE001
+            res[n] = {"error": str(e), "stderr": out.stderr[-500:]}
+        print(n, res[n], flush=True)
+    return res
+
+
+if __name__ == "__main__":
+    names = [a for a in sys.argv[2:] if not a.startswith("--")] or list(VARIANTS)
+    extra = [a for a in sys.argv[2:] if a.startswith("--")]
+    if sys.argv[1] == "build":
+        build(names)
+    else:
+        r = run(names, [x for e in extra for x in e.split("=", 1)])
+        os.makedirs(os.path.join(ROOT, "gpurun_out"), exist_ok=True)
+        with open(os.path.join(ROOT, "gpurun_out", "ab.json"), "w") as fh:
+            json.dump(r, fh, indent=1)
