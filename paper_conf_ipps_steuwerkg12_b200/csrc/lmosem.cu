@@ -37,7 +37,6 @@ struct lmosem_ctx {
     float* c = nullptr;        // error image, bricks (kept all-zero between subsets)
     float* fb = nullptr;       // brick copy of the current f
     float* norm = nullptr;     // s in bricks (halo = 0)
-    int* tab = nullptr;        // per-axis brick index tables (device)
     float* scratch = nullptr;  // V floats, row layout (norm upload)
     int cap = 0;               // path-piece capacity per warp
     size_t proj_smem = 0;      // dynamic shared memory of k_project
@@ -124,11 +123,11 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
     const float* evf = reinterpret_cast<const float*>(ev);
     if (mode == 0)
-        lmk::k_project<0><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, ctx->c, nullptr, ctx->tab,
-                                                                      ctx->geom, ctx->cap);
+        lmk::k_project<0><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, ctx->c, nullptr, ctx->geom,
+                                                                                ctx->cap);
     else
-        lmk::k_project<1><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, nullptr, fp_out, ctx->tab,
-                                                                      ctx->geom, ctx->cap);
+        lmk::k_project<1><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, nullptr, fp_out, ctx->geom,
+                                                                                ctx->cap);
     CK(cudaGetLastError());
     ctx->st.launches++;
     return LMOSEM_OK;
@@ -275,10 +274,6 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
     // padded brick layout: halo of HALO_LO below, >= 2 above, even extents
     for (int k = 0; k < 3; ++k) ctx->geom.P[k] = (dims[k] + 4 + 1) & ~1;
-    ctx->geom.toff[0] = 0;
-    ctx->geom.toff[1] = ctx->geom.P[0];
-    ctx->geom.toff[2] = ctx->geom.P[0] + ctx->geom.P[1];
-    ctx->geom.tsize = ctx->geom.P[0] + ctx->geom.P[1] + ctx->geom.P[2];
     ctx->bricks.BX = ctx->geom.P[0] / 2;
     ctx->bricks.BY = ctx->geom.P[1] / 2;
     ctx->bricks.BZ = ctx->geom.P[2] / 2;
@@ -288,17 +283,17 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         delete ctx;
         return LMOSEM_EINVAL;
     }
-    std::vector<int> tab(ctx->geom.tsize);
     {
         const int64_t M[3] = {8, 8LL * ctx->bricks.BX, 8LL * ctx->bricks.BX * ctx->bricks.BY};
-        const int m[3] = {1, 2, 4};
-        for (int k = 0; k < 3; ++k)
-            for (int p = 0; p < ctx->geom.P[k]; ++p) tab[ctx->geom.toff[k] + p] = (int)(M[k] * (p >> 1) + m[k] * (p & 1));
+        const int64_t m[3] = {1, 2, 4};
+        for (int k = 0; k < 3; ++k) {
+            ctx->geom.A[k] = (int)(M[k] / 2);
+            ctx->geom.B[k] = (int)(m[k] - M[k] / 2);
+        }
     }
-    // <= 3 pieces per dominant-axis slab, + the trash slot
-    ctx->cap = 3 * std::max(dims[0], std::max(dims[1], dims[2])) + 1;
-    ctx->proj_smem = sizeof(int) * (size_t)((ctx->geom.tsize + 1) & ~1) +
-                     (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
+    // <= 3 pieces per dominant-axis slab
+    ctx->cap = 3 * std::max(dims[0], std::max(dims[1], dims[2]));
+    ctx->proj_smem = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
 
     lmosem_status s = LMOSEM_OK;
     auto cuda = [&](cudaError_t e, const char* what) {
@@ -332,14 +327,11 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cuda(cudaMalloc(&ctx->fb, sizeof(float) * ctx->nbf), "cudaMalloc(fb)");
     cuda(cudaMalloc(&ctx->norm, sizeof(float) * ctx->nbf), "cudaMalloc(norm)");
     cuda(cudaMalloc(&ctx->scratch, sizeof(float) * V), "cudaMalloc(scratch)");
-    cuda(cudaMalloc(&ctx->tab, sizeof(int) * tab.size()), "cudaMalloc(tab)");
     for (int k = 0; k < 2; ++k) {
         cuda(cudaEventCreateWithFlags(&ctx->ev_copied[k], cudaEventDisableTiming), "cudaEventCreate");
         cuda(cudaEventCreateWithFlags(&ctx->ev_consumed[k], cudaEventDisableTiming), "cudaEventCreate");
     }
     if (s != LMOSEM_OK) return bail(s);
-    cuda(cudaMemcpyAsync(ctx->tab, tab.data(), sizeof(int) * tab.size(), cudaMemcpyHostToDevice, ctx->stream),
-         "copy tab");
     cuda(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * V, cudaMemcpyDefault, ctx->stream), "copy norm");
     cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * ctx->nbf, ctx->stream), "memset c");
     cuda(cudaMemsetAsync(ctx->fb, 0, sizeof(float) * ctx->nbf, ctx->stream), "memset fb");
@@ -545,7 +537,6 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (ctx->fb) cudaFree(ctx->fb);
     if (ctx->norm) cudaFree(ctx->norm);
     if (ctx->scratch) cudaFree(ctx->scratch);
-    if (ctx->tab) cudaFree(ctx->tab);
     if (ctx->own_stream) cudaStreamDestroy(ctx->own_stream);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     delete ctx;

@@ -11,15 +11,15 @@
 //     minor positions at the slab plane are one 64-bit integer multiply-add and the
 //     crossings are float32 relative to that plane (values in [0,1], ~1e-7 voxel absolute
 //     error wherever the slab lies). The pieces (j, len) are compacted into the warp's
-//     shared-memory path buffer, slab-major;
-//   - pass 2 (forward projection, lines 9-10): lane m reads piece m and gathers f — lanes
-//     hold consecutive pieces of one path, so they share 32-byte sectors of the brick
-//     layout below; warp reduction gives fp;
-//   - pass 3 (back-projection, lines 12-13): lane m issues red.global.add.f32 of
-//     len/fp into c, again sector-coalesced. c stays resident in the 126 MB L2.
+//     shared-memory path buffer in path order; f is gathered for them in the same loop
+//     (the loads of one slab batch complete while the next batch is computed);
+//   - forward projection (lines 9-10): a warp reduction of the gathered f*len gives fp;
+//   - pass 2 (back-projection, lines 12-13): lane m reads piece m and issues
+//     red.global.add.f32 of len/fp into c; lanes hold consecutive pieces of one path, so
+//     they share 32-byte sectors of the brick layout below. c stays resident in L2.
 // Internal image layout ("bricks"): the volume is padded by a halo (2 voxels low, >= 2
 // high, even extents) and stored as 2x2x2 bricks of 8 floats = one 32-byte L2 sector;
-// index J = Tx[px] + Ty[py] + Tz[pz] with T_axis(p) = M_axis*(p>>1) + m_axis*(p&1),
+// index J = Jx(px) + Jy(py) + Jz(pz) with J_axis(p) = M_axis*(p>>1) + m_axis*(p&1),
 // (M, m) = (8, 1), (8*BX, 2), (8*BX*BY, 4). Rounding slivers that step one voxel past
 // the volume land in the halo (f = 0 there, c ignored), so the hot loop has no range
 // checks. Step 2 (lines 16-17 + norm) is k_update over bricks; it also re-zeroes c and
@@ -36,11 +36,13 @@ constexpr int HALO_LO = 2;  // padded coordinate p = i + HALO_LO
 struct GridGeom {
     int n[3];         // nx, ny, nz (real volume)
     int P[3];         // padded extents (even, >= n + 4)
-    int toff[3];      // offsets of the per-axis index tables in the table array
-    int tsize;        // total table entries = P[0] + P[1] + P[2]
+    int A[3], B[3];   // brick index of padded coordinate p on axis k: A[k]*p + B[k]*(p & 1)
     double lo[3];     // volume lower corner (mm): -n*v/2
     double inv_v[3];  // 1 / voxel size (1/mm)
 };
+
+// J_axis(p) = M*(p>>1) + m*(p&1) = (M/2)*p + (m - M/2)*(p&1), (M, m) = (8,1), (8BX,2), (8BX*BY,4)
+__device__ __forceinline__ int bidx(int A, int B, int p) { return A * p + B * (p & 1); }
 
 // Minor-axis positions are fixed point Q24.40 (int64, 2^-40 voxel): exact integer
 // stepping w(k) = w0 + k*s, floor = w >> 40, fraction = low 40 bits. The slope error
@@ -55,7 +57,7 @@ struct Lor {
     float lunit;      // mm of chord per unit of u_a
     float fin, fout;  // clip inside the first / last slab (local coordinate in [0,1])
     int i0, ns;       // first slab index along a, number of slabs
-    int ta, tb, tc;   // table offsets of axes a, b, c, pre-shifted by HALO_LO
+    int Aa, Ba, Ab, Bb, Ac, Bc;  // brick index coefficients of axes a, b, c
     int steps;        // bits 0-1: step of b (+1 -> 1, -1 -> 3, 0 -> 0); bits 2-3: same for c
 };
 
@@ -125,9 +127,9 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     L.fout = fminf(fmaxf((float)(ua_out - (double)il), 0.0f), 1.0f);
     L.i0 = i0;
     L.ns = il - i0 + 1;
-    L.ta = sel3(g.toff, a) + HALO_LO;
-    L.tb = sel3(g.toff, b) + HALO_LO;
-    L.tc = sel3(g.toff, c) + HALO_LO;
+    L.Aa = sel3(g.A, a); L.Ba = sel3(g.B, a);
+    L.Ab = sel3(g.A, b); L.Bb = sel3(g.B, b);
+    L.Ac = sel3(g.A, c); L.Bc = sel3(g.B, c);
     L.steps = (sb > 0.0 ? 1 : (sb < 0.0 ? 3 : 0)) | (sc > 0.0 ? 4 : (sc < 0.0 ? 12 : 0));
     return true;
 }
@@ -171,21 +173,24 @@ __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     L.fout = __shfl_sync(0xffffffffu, s.fout, src);
     L.i0 = __shfl_sync(0xffffffffu, s.i0, src);
     L.ns = __shfl_sync(0xffffffffu, s.ns, src);
-    L.ta = __shfl_sync(0xffffffffu, s.ta, src);
-    L.tb = __shfl_sync(0xffffffffu, s.tb, src);
-    L.tc = __shfl_sync(0xffffffffu, s.tc, src);
+    L.Aa = __shfl_sync(0xffffffffu, s.Aa, src);
+    L.Ba = __shfl_sync(0xffffffffu, s.Ba, src);
+    L.Ab = __shfl_sync(0xffffffffu, s.Ab, src);
+    L.Bb = __shfl_sync(0xffffffffu, s.Bb, src);
+    L.Ac = __shfl_sync(0xffffffffu, s.Ac, src);
+    L.Bc = __shfl_sync(0xffffffffu, s.Bc, src);
     L.steps = __shfl_sync(0xffffffffu, s.steps, src);
     return L;
 }
 
 // The (up to) three pieces of slab k: j = brick index, l = chord length in mm (0 for
-// an empty piece). tab = per-axis brick index tables (shared memory, 2-5 KB).
+// an empty piece).
 struct Pieces {
     int j0, j1, j2;
     float l0, l1, l2;
 };
 
-__device__ __forceinline__ Pieces slab_pieces(const Lor& L, int k, int stb, int stc, const int* __restrict__ tab) {
+__device__ __forceinline__ Pieces slab_pieces(const Lor& L, int k, int stb, int stc) {
     int ib, ic;
     const float gb = fix_to_plane(L.wb0 + (long long)k * L.sb, stb > 0, ib);
     const float gc = fix_to_plane(L.wc0 + (long long)k * L.sc, stc > 0, ic);
@@ -195,9 +200,9 @@ __device__ __forceinline__ Pieces slab_pieces(const Lor& L, int k, int stb, int 
     const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;
     const float q1 = fminf(fmaxf(fminf(db, dc), dlo), dhi);
     const float q2 = fminf(fmaxf(fmaxf(db, dc), dlo), dhi);
-    const int Ja = tab[L.ta + L.i0 + k];
-    const int Jb0 = tab[L.tb + ib], Jb1 = tab[L.tb + ib + stb];
-    const int Jc0 = tab[L.tc + ic], Jc1 = tab[L.tc + ic + stc];
+    const int Ja = bidx(L.Aa, L.Ba, L.i0 + k + HALO_LO);
+    const int Jb0 = bidx(L.Ab, L.Bb, ib + HALO_LO), Jb1 = bidx(L.Ab, L.Bb, ib + HALO_LO + stb);
+    const int Jc0 = bidx(L.Ac, L.Bc, ic + HALO_LO), Jc1 = bidx(L.Ac, L.Bc, ic + HALO_LO + stc);
     // piece 0 before both crossings, piece 2 after both, piece 1 after the first one
     Pieces P;
     P.j0 = Ja + Jb0 + Jc0;
@@ -223,17 +228,18 @@ __device__ __forceinline__ void load_event(const float* __restrict__ events, int
     ev[0] = a.x; ev[1] = a.y; ev[2] = b.x; ev[3] = b.y; ev[4] = c.x; ev[5] = c.y;
 }
 
-// Appends piece (j, l) to the warp's path buffer if v (ballot compaction, slab-major);
-// lanes without a piece store to the warp's trash slot, so the store is unconditional.
-__device__ __forceinline__ void append(int2* __restrict__ path, int trash, int& cnt, unsigned lt, bool v, int j,
-                                       float l) {
-    const unsigned bal = __ballot_sync(0xffffffffu, v);
-#if LMK_TRASH
-    path[v ? cnt + __popc(bal & lt) : trash] = make_int2(j, __float_as_int(l));
-#else
-    if (v) path[cnt + __popc(bal & lt)] = make_int2(j, __float_as_int(l));
-#endif
-    cnt += __popc(bal);
+// Appends the valid pieces of every lane to the warp's path buffer in path order
+// (lane-major = slab order, then piece order): the exclusive prefix of the per-lane
+// counts n = v0 + v1 + v2 (0..3) comes from two ballots on its bits.
+__device__ __forceinline__ void append3(int2* __restrict__ path, int& cnt, unsigned lt, const Pieces& P, bool v0,
+                                        bool v1, bool v2) {
+    const int n = (int)v0 + (int)v1 + (int)v2;
+    const unsigned b0 = __ballot_sync(0xffffffffu, n & 1), b1 = __ballot_sync(0xffffffffu, n & 2);
+    const int pos = cnt + __popc(b0 & lt) + 2 * __popc(b1 & lt);
+    if (v0) path[pos] = make_int2(P.j0, __float_as_int(P.l0));
+    if (v1) path[pos + v0] = make_int2(P.j1, __float_as_int(P.l1));
+    if (v2) path[pos + v0 + v1] = make_int2(P.j2, __float_as_int(P.l2));
+    cnt += __popc(b0) + 2 * __popc(b1);
 }
 
 #ifndef LMK_CTA_THREADS
@@ -242,32 +248,22 @@ __device__ __forceinline__ void append(int2* __restrict__ path, int trash, int& 
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
-#ifndef LMK_TRASH
-#define LMK_TRASH 0          // 1: unconditional store to a trash slot; 0: predicated store
-#endif
 #ifndef LMK_FUSED_GATHER
 #define LMK_FUSED_GATHER 1   // 1: gather f during the geometry pass (no separate pass 2)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 
-// Dynamic shared memory: int tab[tsize] (rounded up to 8 B), then per warp `cap` path
-// pieces (int j, float len) packed as int2; the last one is the warp's trash slot.
+// Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2.
 // MODE 0: fused forward + back-projection into cb (step 1).
 // MODE 1: forward projection only, fp written to fp_out[i] (tests).
 template <int MODE>
 __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
-                                                             float* __restrict__ fp_out, const int* __restrict__ tab_g,
-                                                             GridGeom g, int cap) {
-    extern __shared__ __align__(16) int smem[];
-    int* tab = smem;
-    const int tpad = (g.tsize + 1) & ~1;
-    for (int t = threadIdx.x; t < g.tsize; t += blockDim.x) tab[t] = tab_g[t];
-    __syncthreads();
+                                                             float* __restrict__ fp_out, GridGeom g, int cap) {
+    extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
-    int2* path = reinterpret_cast<int2*>(smem + tpad) + (size_t)wib * cap;
-    const int trash = cap - 1;
+    int2* path = smem_path + (size_t)wib * cap;
     const unsigned lt = (1u << lane) - 1u;
     const int64_t warp = (int64_t)blockIdx.x * (blockDim.x >> 5) + wib;
     const int64_t nwarps = (int64_t)gridDim.x * (blockDim.x >> 5);
@@ -298,11 +294,9 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
             float g0 = 0.f, g1 = 0.f, g2 = 0.f, w0 = 0.f, w1 = 0.f, w2 = 0.f;
             for (int k0 = 0; k0 < L.ns; k0 += 32) {
                 const bool in = k0 + lane < L.ns;
-                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc, tab);
+                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
-                append(path, trash, cnt, lt, v0, P.j0, P.l0);
-                append(path, trash, cnt, lt, v1, P.j1, P.l1);
-                append(path, trash, cnt, lt, v2, P.j2, P.l2);
+                append3(path, cnt, lt, P, v0, v1, v2);
                 acc = fmaf(g0, w0, acc);
                 acc = fmaf(g1, w1, acc);
                 acc = fmaf(g2, w2, acc);
@@ -318,10 +312,8 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
 #else
             for (int k0 = 0; k0 < L.ns; k0 += 32) {
                 const bool in = k0 + lane < L.ns;
-                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc, tab);
-                append(path, trash, cnt, lt, in && P.l0 > 0.0f, P.j0, P.l0);
-                append(path, trash, cnt, lt, in && P.l1 > 0.0f, P.j1, P.l1);
-                append(path, trash, cnt, lt, in && P.l2 > 0.0f, P.j2, P.l2);
+                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
+                append3(path, cnt, lt, P, in && P.l0 > 0.0f, in && P.l1 > 0.0f, in && P.l2 > 0.0f);
             }
             __syncwarp();
             // pass 2: forward projection, lane m <- piece m
