@@ -107,6 +107,17 @@ lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
 lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
                           const float* norm, const lmosem_dist* dist);
 
+/* Out-of-L2 strategy: step 1 runs as z-slab passes when the
+ * image is too large for L2 — pass A accumulates each event's forward projection over
+ * slabs of the volume, pass B back-projects slab by slab with the complete fp — so each
+ * launch touches one L2-sized image slab. n_slabs = 0 (default) picks the count from a
+ * 48 MB-per-slab L2 budget (1 = single fused pass); n_slabs > 0 forces it (clamped to
+ * nz/2). The result is the same up to fp32 rounding. EINVAL if n_slabs < 0. */
+lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs);
+
+/* The z-slab count step 1 currently uses (-1 for a NULL context). */
+int32_t lmosem_get_slabs(const lmosem_ctx* ctx);
+
 /* Uses the given cudaStream_t (as void*) for all later device work; NULL means the CUDA
  * default stream (torch's default stream is NULL). Until this is called the context uses
  * its own non-blocking stream. The stream must belong to the context's device. */

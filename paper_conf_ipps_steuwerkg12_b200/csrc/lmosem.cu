@@ -39,6 +39,9 @@ struct lmosem_ctx {
     float* norm = nullptr;     // s in bricks (halo = 0)
     float* scratch = nullptr;  // V floats, row layout (norm upload)
     int cap = 0;               // path-piece capacity per warp
+    int slabs_forced = 0;      // z-slab count (0 = automatic from the L2 budget)
+    float* fp_acc = nullptr;   // per-event forward projections of the z-slab passes
+    int64_t fp_cap = 0;
     size_t proj_smem = 0;      // dynamic shared memory of k_project
     cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
     int rank = 0, world = 1;
@@ -113,23 +116,59 @@ lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
     return LMOSEM_OK;
 }
 
-// k_project over n device events against ctx->fb; mode 0 accumulates into ctx->c.
-lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* fp_out, int mode) {
-    if (n <= 0) return LMOSEM_OK;
+// Number of z-slabs for the projection: the brick image must stay L2-resident during a
+// pass (L2 126 MB; budget 48 MB per image slab leaves room for the event stream and the
+// per-event fp array). 1 = the single fused pass.
+int n_slabs(const lmosem_ctx* ctx) {
+    const int max_slabs = std::max(1, ctx->dims[2] / 2);
+    if (ctx->slabs_forced > 0) return std::min(ctx->slabs_forced, max_slabs);
+    const double bytes = 4.0 * (double)ctx->nbf;
+    const double budget = 48.0 * 1024 * 1024;
+    return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
+}
+
+lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
     const int64_t warps_needed = (n + 31) / 32;
     const int64_t wpb = lmk::PROJ_THREADS / 32;
     const int64_t blocks_needed = (warps_needed + wpb - 1) / wpb;
     const int64_t cap = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm;
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
-    const float* evf = reinterpret_cast<const float*>(ev);
-    if (mode == 0)
-        lmk::k_project<0><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, ctx->c, nullptr, ctx->geom,
-                                                                                ctx->cap);
-    else
-        lmk::k_project<1><<<grid, lmk::PROJ_THREADS, ctx->proj_smem, ctx->stream>>>(evf, n, ctx->fb, nullptr, fp_out, ctx->geom,
-                                                                                ctx->cap);
+    const size_t sm = ctx->proj_smem;
+    switch (mode) {
+        case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+        case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+        case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+        default: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+    }
     CK(cudaGetLastError());
     ctx->st.launches++;
+    return LMOSEM_OK;
+}
+
+// Step 1 over n device events against ctx->fb (mode 0: accumulate into ctx->c; mode 1:
+// forward projections into fp_out). Large images run the z-slab two-pass form.
+lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* fp_out, int mode) {
+    if (n <= 0) return LMOSEM_OK;
+    const float* evf = reinterpret_cast<const float*>(ev);
+    const int K = n_slabs(ctx);
+    if (mode == 1 || K == 1) return launch_mode(ctx, mode, evf, n, fp_out, ctx->geom);
+    if (n > ctx->fp_cap) {
+        if (ctx->fp_acc) CK(cudaFree(ctx->fp_acc));
+        ctx->fp_acc = nullptr;
+        ctx->fp_cap = 0;
+        CK(cudaMalloc(&ctx->fp_acc, sizeof(float) * n));
+        ctx->fp_cap = n;
+    }
+    CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
+    const int half = ctx->dims[2] / 2;  // slab boundaries on even z (brick aligned)
+    lmosem_status s;
+    for (int pass = 2; pass <= 3; ++pass)
+        for (int k = 0; k < K; ++k) {
+            lmk::GridGeom g = ctx->geom;
+            g.clo[2] = 2 * (int)((int64_t)half * k / K);
+            g.chi[2] = (k == K - 1) ? ctx->dims[2] : 2 * (int)((int64_t)half * (k + 1) / K);
+            if ((s = launch_mode(ctx, pass, evf, n, ctx->fp_acc, g))) return s;
+        }
     return LMOSEM_OK;
 }
 
@@ -220,7 +259,7 @@ lmosem_status resolve_timing(lmosem_ctx* ctx) {
 
 }  // namespace
 
-LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.2 sm_100a"; }
+LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.3 sm_100a"; }
 
 LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end) {
     if (!begin || !end || n < 0 || world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
@@ -272,6 +311,10 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         ctx->geom.lo[k] = -0.5 * (double)dims[k] * (double)voxel_mm[k];
         ctx->geom.inv_v[k] = 1.0 / (double)voxel_mm[k];
     }
+    for (int k = 0; k < 3; ++k) {
+        ctx->geom.clo[k] = 0;
+        ctx->geom.chi[k] = dims[k];
+    }
     // padded brick layout: halo of HALO_LO below, >= 2 above, even extents
     for (int k = 0; k < 3; ++k) ctx->geom.P[k] = (dims[k] + 4 + 1) & ~1;
     ctx->bricks.BX = ctx->geom.P[0] / 2;
@@ -311,9 +354,15 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         ctx->err = "volume too large for the shared-memory path buffer";
         return bail(LMOSEM_EINVAL);
     }
+
+
     cuda(cudaFuncSetAttribute(lmk::k_project<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
          "smem attr");
     cuda(cudaFuncSetAttribute(lmk::k_project<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
+         "smem attr");
+    cuda(cudaFuncSetAttribute(lmk::k_project<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
+         "smem attr");
+    cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
          "smem attr");
     cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, lmk::PROJ_THREADS,
                                                        ctx->proj_smem),
@@ -355,6 +404,15 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     *out = ctx;
     return LMOSEM_OK;
 }
+
+LMOSEM_API lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs) {
+    USABLE(ctx);
+    if (n_slabs < 0) return fail(ctx, LMOSEM_EINVAL, "set_slabs: n_slabs < 0");
+    ctx->slabs_forced = n_slabs;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API int32_t lmosem_get_slabs(const lmosem_ctx* ctx) { return ctx ? n_slabs(ctx) : -1; }
 
 LMOSEM_API lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream) {
     USABLE(ctx);
@@ -537,6 +595,7 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (ctx->fb) cudaFree(ctx->fb);
     if (ctx->norm) cudaFree(ctx->norm);
     if (ctx->scratch) cudaFree(ctx->scratch);
+    if (ctx->fp_acc) cudaFree(ctx->fp_acc);
     if (ctx->own_stream) cudaStreamDestroy(ctx->own_stream);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     delete ctx;

@@ -37,6 +37,7 @@ struct GridGeom {
     int n[3];         // nx, ny, nz (real volume)
     int P[3];         // padded extents (even, >= n + 4)
     int A[3], B[3];   // brick index of padded coordinate p on axis k: A[k]*p + B[k]*(p & 1)
+    int clo[3], chi[3];  // clip box in voxels: [0, n) except z = [zlo, zhi) of a z-slab pass
     double lo[3];     // volume lower corner (mm): -n*v/2
     double inv_v[3];  // 1 / voxel size (1/mm)
 };
@@ -86,12 +87,13 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     double amin = 0.0, amax = 1.0;
 #pragma unroll
     for (int k = 0; k < 3; ++k) {
+        const double lo = (double)g.clo[k], hi = (double)g.chi[k];
         if (D[k] != 0.0) {
             double r = 1.0 / D[k];
-            double t0 = -u1[k] * r, t1 = ((double)g.n[k] - u1[k]) * r;
+            double t0 = (lo - u1[k]) * r, t1 = (hi - u1[k]) * r;
             amin = fmax(amin, fmin(t0, t1));
             amax = fmin(amax, fmax(t0, t1));
-        } else if (u1[k] < 0.0 || u1[k] >= (double)g.n[k]) {
+        } else if (u1[k] < lo || u1[k] >= hi) {
             return false;
         }
     }
@@ -104,9 +106,8 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     const double Db = sel3(D, b), Dc = sel3(D, c), u1b = sel3(u1, b), u1c = sel3(u1, c);
     double ua_in = u1a + amin * Da, ua_out = u1a + amax * Da;
     if (Da < 0.0) { double t = ua_in; ua_in = ua_out; ua_out = t; }
-    const int na = sel3(g.n, a);
-    int i0 = max((int)floor(ua_in), 0);
-    int il = min((int)ceil(ua_out) - 1, na - 1);
+    int i0 = max((int)floor(ua_in), sel3(g.clo, a));
+    int il = min((int)ceil(ua_out) - 1, sel3(g.chi, a) - 1);
     if (il < i0) return false;
     const double rDa = 1.0 / Da;
     const double sb = Db * rDa, sc = Dc * rDa;
@@ -248,18 +249,22 @@ __device__ __forceinline__ void append3(int2* __restrict__ path, int& cnt, unsig
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
-#ifndef LMK_FUSED_GATHER
-#define LMK_FUSED_GATHER 1   // 1: gather f during the geometry pass (no separate pass 2)
-#endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 
 // Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2.
-// MODE 0: fused forward + back-projection into cb (step 1).
-// MODE 1: forward projection only, fp written to fp_out[i] (tests).
+// MODE 0: fused forward + back-projection into cb (step 1, image resident in L2).
+// MODE 1: forward projection only, fp[i] = fp (tests).
+// MODE 2: z-slab pass A: fp[i] += forward projection of the part of LOR i in the slab.
+// MODE 3: z-slab pass B: back-projection of the slab part of LOR i with the complete
+//         fp[i] from pass A (events with fp <= 0 skipped).
+// MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
+// L2-sized slab of the image.
 template <int MODE>
 __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
-                                                             float* __restrict__ fp_out, GridGeom g, int cap) {
+                                                             float* __restrict__ fp, GridGeom g, int cap) {
+    constexpr bool kGather = MODE != 3;    // forward projection in this launch
+    constexpr bool kScatter = MODE == 0 || MODE == 3;  // back-projection in this launch
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
@@ -271,12 +276,17 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
         const int64_t idx = base + lane;
         Lor mine;
         bool ok = false;
+        float fp_known = 0.0f;
         if (idx < n) {
             float ev[6];
             load_event(events, idx, ev);
             ok = lor_setup(ev, g, mine);
+            if (MODE == 3) {
+                fp_known = fp[idx];
+                ok = ok && fp_known > 0.0f;  // reading S7
+            }
         }
-        if (MODE == 1 && idx < n && !ok) fp_out[idx] = 0.0f;
+        if (MODE == 1 && idx < n && !ok) fp[idx] = 0.0f;
         unsigned mask = __ballot_sync(0xffffffffu, ok);
         while (mask) {
             const int src = __ffs(mask) - 1;
@@ -284,51 +294,44 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
             const Lor L = shfl_lor(mine, src);
             const int stb = ((L.steps & 3) == 1) - ((L.steps & 3) == 3);
             const int stc = ((L.steps & 12) == 4) - ((L.steps & 12) == 12);
-            // pass 1: geometry -> compacted path pieces in shared memory (uniform loop:
-            // lanes past the last slab recompute it and drop their pieces)
+            // pass 1: geometry (uniform loop: lanes past the last slab recompute it and drop
+            // their pieces) -> path pieces in shared memory (when back-projecting) and f
+            // gathered in the same loop (when forward-projecting): each iteration consumes
+            // the previous iteration's loads, so their latency overlaps the next batch
             int cnt = 0;
             float acc = 0.0f;
-#if LMK_FUSED_GATHER
-            // gathers issued with the geometry; each iteration consumes the previous
-            // iteration's loads, so their latency overlaps the next slab batch
             float g0 = 0.f, g1 = 0.f, g2 = 0.f, w0 = 0.f, w1 = 0.f, w2 = 0.f;
             for (int k0 = 0; k0 < L.ns; k0 += 32) {
                 const bool in = k0 + lane < L.ns;
                 const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
-                append3(path, cnt, lt, P, v0, v1, v2);
+                if (kScatter) append3(path, cnt, lt, P, v0, v1, v2);
+                if (kGather) {
+                    acc = fmaf(g0, w0, acc);
+                    acc = fmaf(g1, w1, acc);
+                    acc = fmaf(g2, w2, acc);
+                    g0 = v0 ? __ldg(fb + P.j0) : 0.f;
+                    g1 = v1 ? __ldg(fb + P.j1) : 0.f;
+                    g2 = v2 ? __ldg(fb + P.j2) : 0.f;
+                    w0 = P.l0; w1 = P.l1; w2 = P.l2;
+                }
+            }
+            float fpv = fp_known;
+            if (kGather) {
                 acc = fmaf(g0, w0, acc);
                 acc = fmaf(g1, w1, acc);
                 acc = fmaf(g2, w2, acc);
-                g0 = v0 ? __ldg(fb + P.j0) : 0.f;
-                g1 = v1 ? __ldg(fb + P.j1) : 0.f;
-                g2 = v2 ? __ldg(fb + P.j2) : 0.f;
-                w0 = P.l0; w1 = P.l1; w2 = P.l2;
-            }
-            acc = fmaf(g0, w0, acc);
-            acc = fmaf(g1, w1, acc);
-            acc = fmaf(g2, w2, acc);
-            __syncwarp();
-#else
-            for (int k0 = 0; k0 < L.ns; k0 += 32) {
-                const bool in = k0 + lane < L.ns;
-                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
-                append3(path, cnt, lt, P, in && P.l0 > 0.0f, in && P.l1 > 0.0f, in && P.l2 > 0.0f);
+                fpv = warp_sum(acc);
+                if (MODE == 1 && lane == 0) fp[base + src] = fpv;
+                if (MODE == 2 && lane == 0) fp[base + src] += fpv;
+            } else {
+                fpv = __shfl_sync(0xffffffffu, fp_known, src);
             }
             __syncwarp();
-            // pass 2: forward projection, lane m <- piece m
-#pragma unroll 8
-            for (int m = lane; m < cnt; m += 32) {
-                const int2 q = path[m];
-                acc = fmaf(__ldg(fb + q.x), __int_as_float(q.y), acc);
-            }
-#endif
-            const float fp = warp_sum(acc);
-            if (MODE == 1) {
-                if (lane == 0) fp_out[base + src] = fp;
-            } else if (fp > 0.0f) {  // reading S7: skip events with fp <= 0
-                // pass 3: back-projection
-                const float inv = 1.0f / fp;
+            if (kScatter && fpv > 0.0f) {  // reading S7: skip events with fp <= 0
+                // pass 2: back-projection, lane m <- piece m (path order: consecutive
+                // lanes share 32-byte brick sectors)
+                const float inv = 1.0f / fpv;
 #pragma unroll 8
                 for (int m = lane; m < cnt; m += 32) {
                     const int2 q = path[m];

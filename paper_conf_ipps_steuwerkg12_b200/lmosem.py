@@ -25,7 +25,7 @@ EXPORTS = (
     "lmosem_version", "lmosem_block_range", "lmosem_nccl_unique_id", "lmosem_init", "lmosem_set_stream",
     "lmosem_subset_step", "lmosem_reconstruct", "lmosem_reconstruct_host", "lmosem_error_image",
     "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
-    "lmosem_destroy", "lmosem_last_error",
+    "lmosem_destroy", "lmosem_last_error", "lmosem_set_slabs", "lmosem_get_slabs",
 )
 
 
@@ -72,6 +72,8 @@ def load(build_if_missing: bool = False) -> ctypes.CDLL:
         "lmosem_nccl_unique_id": ([_P, ctypes.c_size_t], _S),
         "lmosem_init": ([ctypes.POINTER(_P), _P, _P, _P, ctypes.POINTER(Dist)], _S),
         "lmosem_set_stream": ([_P, _P], _S),
+        "lmosem_set_slabs": ([_P, _I32], _S),
+        "lmosem_get_slabs": ([_P], _I32),
         "lmosem_subset_step": ([_P, _P, _I64, _P], _S),
         "lmosem_reconstruct": ([_P, _P, _P, _I32, _I32, _P], _S),
         "lmosem_reconstruct_host": ([_P, _P, _P, _I32, _I32, _P], _S),
@@ -244,6 +246,14 @@ class Reconstructor:
 
     def update(self, f, c):
         self._check(self._lib.lmosem_update(self._h, _dev_ptr(f, "float32", self.V), _dev_ptr(c, "float32", self.V)))
+
+    def set_slabs(self, n_slabs: int):
+        """z-slab passes for step 1 (0 = automatic from the L2 budget); see lmosem.h."""
+        self._check(self._lib.lmosem_set_slabs(self._h, int(n_slabs)))
+
+    @property
+    def slabs(self) -> int:
+        return int(self._lib.lmosem_get_slabs(self._h))
 
     def synchronize(self):
         self._check(self._lib.lmosem_synchronize(self._h))

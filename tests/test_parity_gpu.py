@@ -289,6 +289,7 @@ def test_c4_full_size_properties(pkg):
     s = lmgen.norm(cfg)
     g = oracle.geom(cfg.dims, cfg.voxel_mm)
     rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    assert rec.slabs > 1  # 200 MB images: the z-slab (out-of-L2) form runs
     f0 = np.ones(cfg.n_voxels, np.float32)
     evd = dev(ev)
     # sampled forward projections
@@ -315,3 +316,38 @@ def test_c4_full_size_properties(pkg):
     assert np.all(got > 0) and np.all(got[~hit] == 1.0)
     assert torch.count_nonzero(c).item() == 0  # the update re-zeroes c
     rec.close()
+
+
+# ------------------------------------------------------------------ z-slab (out-of-L2) form
+@pytest.mark.parametrize("slabs", [2, 3, 5])
+def test_zslab_passes_match_oracle_c1(pkg, slabs):
+    """The z-slab two-pass form of step 1 (pass A: per-slab partial forward projections,
+    pass B: per-slab back-projection with the complete fp) gives the oracle's subset."""
+    cfg, ev, s = inputs("C1")
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    rec.set_slabs(slabs)
+    assert rec.slabs == slabs
+    f0 = np.random.default_rng(11).uniform(0.5, 2.0, cfg.n_voxels)
+    f = dev(f0.astype(np.float32))
+    rec.subset_step(dev(ev[:cfg.n_events]), f)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    rec.close()
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], s, f0.astype(np.float32))
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+def test_zslab_passes_match_oracle_c2(pkg):
+    cfg = lmgen.CONFIGS["C2"]
+    ev = lmgen.subset_events(cfg, 3)
+    s = lmgen.norm(cfg)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    assert rec.slabs == 1  # 27 MB brick image: single fused pass
+    rec.set_slabs(4)
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.subset_step(dev(ev), f)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    rec.close()
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev, s, np.ones(cfg.n_voxels))
+    assert maxrel(got, ref) <= MAXREL_SUBSET
