@@ -16,7 +16,9 @@ enum {
     L2PEAK_LDG_RANDOM = 1,    /* fp32 gathers at uniformly random addresses */
     L2PEAK_PAIR_RANDOM = 2,   /* one gather + one red per op (the projection's mix) */
     L2PEAK_RED_RUN8 = 3,      /* red where each 8 lanes hit 8 consecutive floats */
-    L2PEAK_PAIR_RUN8 = 4      /* gather + red, 8-lane runs */
+    L2PEAK_PAIR_RUN8 = 4,     /* gather + red, 8-lane runs */
+    L2PEAK_PAIR_WARP32 = 5    /* gather + red, each warp on 32 consecutive floats (fully
+                                 coalesced: the L2 peak for this op mix) */
 };
 
 /* Runs `mode` on the current device over a buffer of n_floats floats (device memory

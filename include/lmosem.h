@@ -150,6 +150,17 @@ lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event* events, in
 lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
                              const float* f, float* fp_out);
 
+/* Sensitivity (norm) image over a set of LORs (the norm image of
+ * BASELINE.json north_star): s_out_j = sum_i a_ij, the back-projection of ones with the
+ * same exact traversal as step 1 (no forward projection). s_out: V float32 device,
+ * x-fastest, overwritten. Collective with world > 1 (block split + all-reduce, every rank
+ * gets the full image). Stream-ordered. */
+lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events, float* s_out);
+
+/* Replaces the context's norm image s (V float32, device or host; copied). Stream-ordered:
+ * later calls use the new s. EINVAL for NULL. */
+lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm);
+
 /* Step 2 only, for tests: f_j <- f_j*c_j/s_j where c_j > 0 and s_j > 0 (device f and c,
  * both V float32 x-fastest; the context's norm); c is re-zeroed. */
 lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c);

@@ -58,6 +58,7 @@ def _load():
         lib.oracle_forward.argtypes = [G, _P, ctypes.c_int64, _P, _P]
         lib.oracle_error_image.argtypes = [G, _P, ctypes.c_int64, _P, _P]
         lib.oracle_update.argtypes = [ctypes.c_int64, _P, _P, _P]
+        lib.oracle_sensitivity.argtypes = [G, _P, ctypes.c_int64, _P]
         lib.oracle_subset_step.argtypes = [G, _P, ctypes.c_int64, _P, _P]
         lib.oracle_subset_step.restype = ctypes.c_int
         lib.oracle_reconstruct.argtypes = [G, _P, _P, ctypes.c_int32, ctypes.c_int32, _P, _P]
@@ -114,6 +115,14 @@ def error_image(g: Geom, events, f) -> np.ndarray:
     c = np.empty(int(g.nx) * g.ny * g.nz, np.float64)
     _load().oracle_error_image(ctypes.byref(g), ev.ctypes.data, ev.shape[0], f.ctypes.data, c.ctypes.data)
     return c
+
+
+def sensitivity(g: Geom, events) -> np.ndarray:
+    """s_j = sum_i a_ij over the given LORs (back-projection of ones), float64[V]."""
+    ev = _f32(events).reshape(-1, 6)
+    out = np.empty(int(g.nx) * g.ny * g.nz, np.float64)
+    _load().oracle_sensitivity(ctypes.byref(g), ev.ctypes.data, ev.shape[0], out.ctypes.data)
+    return out
 
 
 def update(f, c, s) -> np.ndarray:

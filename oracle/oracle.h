@@ -53,6 +53,10 @@ void oracle_forward(const oracle_geom* g, const float* events, int64_t n, const 
 /* Error image (step 1, Listing 2 lines 5-13) for n events; c is zeroed first (S8). */
 void oracle_error_image(const oracle_geom* g, const float* events, int64_t n, const double* f, double* c);
 
+/* Sensitivity image s_j = sum_i a_ij over n LORs (the back-projection of ones; the norm
+ * image of BASELINE.json north_star). s is zeroed first. */
+void oracle_sensitivity(const oracle_geom* g, const float* events, int64_t n, double* s);
+
 /* Image update (step 2, Listing 2 lines 16-17, with the norm of BASELINE.json north_star):
  * f_j <- f_j * c_j / s_j if c_j > 0 and s_j > 0, else unchanged (S9). */
 void oracle_update(int64_t V, double* f, const double* c, const float* s);

@@ -138,20 +138,36 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
         case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
         case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
         case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
-        default: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+        case 3: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+        default: lmk::k_project<4><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
     }
     CK(cudaGetLastError());
     ctx->st.launches++;
     return LMOSEM_OK;
 }
 
+lmk::GridGeom slab_geom(const lmosem_ctx* ctx, int k, int K) {
+    const int half = ctx->dims[2] / 2;  // slab boundaries on even z (brick aligned)
+    lmk::GridGeom g = ctx->geom;
+    g.clo[2] = 2 * (int)((int64_t)half * k / K);
+    g.chi[2] = (k == K - 1) ? ctx->dims[2] : 2 * (int)((int64_t)half * (k + 1) / K);
+    return g;
+}
+
 // Step 1 over n device events against ctx->fb (mode 0: accumulate into ctx->c; mode 1:
-// forward projections into fp_out). Large images run the z-slab two-pass form.
+// forward projections into fp_out; mode 4: sensitivity into ctx->c). Large images run
+// the z-slab form (modes 0 -> 2 + 3; mode 4 slab by slab).
 lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* fp_out, int mode) {
     if (n <= 0) return LMOSEM_OK;
     const float* evf = reinterpret_cast<const float*>(ev);
     const int K = n_slabs(ctx);
     if (mode == 1 || K == 1) return launch_mode(ctx, mode, evf, n, fp_out, ctx->geom);
+    lmosem_status s;
+    if (mode == 4) {
+        for (int k = 0; k < K; ++k)
+            if ((s = launch_mode(ctx, 4, evf, n, nullptr, slab_geom(ctx, k, K)))) return s;
+        return LMOSEM_OK;
+    }
     if (n > ctx->fp_cap) {
         if (ctx->fp_acc) CK(cudaFree(ctx->fp_acc));
         ctx->fp_acc = nullptr;
@@ -160,15 +176,9 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         ctx->fp_cap = n;
     }
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
-    const int half = ctx->dims[2] / 2;  // slab boundaries on even z (brick aligned)
-    lmosem_status s;
     for (int pass = 2; pass <= 3; ++pass)
-        for (int k = 0; k < K; ++k) {
-            lmk::GridGeom g = ctx->geom;
-            g.clo[2] = 2 * (int)((int64_t)half * k / K);
-            g.chi[2] = (k == K - 1) ? ctx->dims[2] : 2 * (int)((int64_t)half * (k + 1) / K);
-            if ((s = launch_mode(ctx, pass, evf, n, ctx->fp_acc, g))) return s;
-        }
+        for (int k = 0; k < K; ++k)
+            if ((s = launch_mode(ctx, pass, evf, n, ctx->fp_acc, slab_geom(ctx, k, K)))) return s;
     return LMOSEM_OK;
 }
 
@@ -364,6 +374,8 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
          "smem attr");
     cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
          "smem attr");
+    cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
+         "smem attr");
     cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, lmk::PROJ_THREADS,
                                                        ctx->proj_smem),
          "occupancy");
@@ -527,6 +539,26 @@ LMOSEM_API lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* eve
     lmosem_status s;
     if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
     return launch_project(ctx, events, n_events, fp_out, 1);
+}
+
+LMOSEM_API lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
+                                            float* s_out) {
+    USABLE(ctx);
+    if (!s_out || n_events < 0 || (n_events > 0 && !events))
+        return fail(ctx, LMOSEM_EINVAL, "sensitivity: bad arguments");
+    int64_t b = 0, e = n_events;
+    block_range(n_events, ctx->rank, ctx->world, &b, &e);
+    lmosem_status s;
+    if ((s = launch_project(ctx, events + b, e - b, nullptr, 4))) return s;
+    if (ctx->world > 1) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    return launch_to_row(ctx, ctx->c, s_out, 1);  // s_out <- c, c <- 0
+}
+
+LMOSEM_API lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm) {
+    USABLE(ctx);
+    if (!norm) return fail(ctx, LMOSEM_EINVAL, "set_norm: null norm");
+    CK(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * ctx->V, cudaMemcpyDefault, ctx->stream));
+    return launch_to_brick(ctx, ctx->scratch, ctx->norm);
 }
 
 LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {

@@ -249,6 +249,9 @@ __device__ __forceinline__ void append3(int2* __restrict__ path, int& cnt, unsig
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
+#ifndef LMK_RECOMPUTE
+#define LMK_RECOMPUTE 0      // 1: back-projection recomputes the geometry (no shared path buffer)
+#endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 
 // Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2.
@@ -257,14 +260,17 @@ constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 // MODE 2: z-slab pass A: fp[i] += forward projection of the part of LOR i in the slab.
 // MODE 3: z-slab pass B: back-projection of the slab part of LOR i with the complete
 //         fp[i] from pass A (events with fp <= 0 skipped).
+// MODE 4: sensitivity image: back-projection of ones, cb_j += a_ij (no forward
+//         projection).
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
 template <int MODE>
 __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap) {
-    constexpr bool kGather = MODE != 3;    // forward projection in this launch
-    constexpr bool kScatter = MODE == 0 || MODE == 3;  // back-projection in this launch
+    constexpr bool kGather = MODE <= 2;    // forward projection in this launch
+    constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4;  // back-projection in this launch
+    constexpr bool kStore = kScatter && !LMK_RECOMPUTE;  // keep pieces for the scatter pass
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
@@ -276,7 +282,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
         const int64_t idx = base + lane;
         Lor mine;
         bool ok = false;
-        float fp_known = 0.0f;
+        float fp_known = 1.0f;  // MODE 4 back-projects len * 1
         if (idx < n) {
             float ev[6];
             load_event(events, idx, ev);
@@ -305,7 +311,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 const bool in = k0 + lane < L.ns;
                 const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
-                if (kScatter) append3(path, cnt, lt, P, v0, v1, v2);
+                if (kStore) append3(path, cnt, lt, P, v0, v1, v2);
                 if (kGather) {
                     acc = fmaf(g0, w0, acc);
                     acc = fmaf(g1, w1, acc);
@@ -332,10 +338,20 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 // pass 2: back-projection, lane m <- piece m (path order: consecutive
                 // lanes share 32-byte brick sectors)
                 const float inv = 1.0f / fpv;
+                if (kStore) {
 #pragma unroll 8
-                for (int m = lane; m < cnt; m += 32) {
-                    const int2 q = path[m];
-                    atomicAdd(cb + q.x, __int_as_float(q.y) * inv);
+                    for (int m = lane; m < cnt; m += 32) {
+                        const int2 q = path[m];
+                        atomicAdd(cb + q.x, __int_as_float(q.y) * inv);
+                    }
+                } else {
+                    for (int k0 = 0; k0 < L.ns; k0 += 32) {
+                        const bool in = k0 + lane < L.ns;
+                        const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
+                        if (in && P.l0 > 0.0f) atomicAdd(cb + P.j0, P.l0 * inv);
+                        if (in && P.l1 > 0.0f) atomicAdd(cb + P.j1, P.l1 * inv);
+                        if (in && P.l2 > 0.0f) atomicAdd(cb + P.j2, P.l2 * inv);
+                    }
                 }
             }
             __syncwarp();

@@ -26,6 +26,7 @@ EXPORTS = (
     "lmosem_subset_step", "lmosem_reconstruct", "lmosem_reconstruct_host", "lmosem_error_image",
     "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
     "lmosem_destroy", "lmosem_last_error", "lmosem_set_slabs", "lmosem_get_slabs",
+    "lmosem_sensitivity", "lmosem_set_norm",
 )
 
 
@@ -80,6 +81,8 @@ def load(build_if_missing: bool = False) -> ctypes.CDLL:
         "lmosem_error_image": ([_P, _P, _I64, _P, _P], _S),
         "lmosem_forward": ([_P, _P, _I64, _P, _P], _S),
         "lmosem_update": ([_P, _P, _P], _S),
+        "lmosem_sensitivity": ([_P, _P, _I64, _P], _S),
+        "lmosem_set_norm": ([_P, _P], _S),
         "lmosem_synchronize": ([_P], _S),
         "lmosem_set_timing": ([_P, _I32], _S),
         "lmosem_get_stats": ([_P, ctypes.POINTER(Stats)], _S),
@@ -243,6 +246,22 @@ class Reconstructor:
         ep, n = self._events_ptr(events)
         self._check(self._lib.lmosem_forward(self._h, ep, n, _dev_ptr(f, "float32", self.V),
                                              _dev_ptr(fp_out, "float32", n) if n else 0))
+
+    def sensitivity(self, events, s_out):
+        """s_out_j = sum_i a_ij over the given LORs (back-projection of ones)."""
+        ep, n = self._events_ptr(events)
+        self._check(self._lib.lmosem_sensitivity(self._h, ep, n, _dev_ptr(s_out, "float32", self.V)))
+
+    def set_norm(self, norm):
+        """Replaces the norm image (CUDA tensor or host float32 array, V elements)."""
+        import torch
+        if isinstance(norm, torch.Tensor) and norm.is_cuda:
+            ptr = _dev_ptr(norm, "float32", self.V)
+        else:
+            ptr = _host_ptr(norm, self.V)
+        self._check(self._lib.lmosem_set_norm(self._h, ptr))
+        if not (isinstance(norm, torch.Tensor) and norm.is_cuda):
+            self.synchronize()  # the host buffer may be released by the caller
 
     def update(self, f, c):
         self._check(self._lib.lmosem_update(self._h, _dev_ptr(f, "float32", self.V), _dev_ptr(c, "float32", self.V)))

@@ -366,3 +366,28 @@ def test_degenerate_events_contribute_nothing():
                   np.float32)
     c = oracle.error_image(g, ev, np.ones(512))
     assert np.all(c == 0)
+
+
+# ---------------------------------------------------------------- P14 sensitivity image
+def test_p14_sensitivity_textbook_and_sum():
+    """s = A^T 1 with A from the brute-force clip (scipy.sparse), and sum_j s_j equals the
+    sum of the chords found by bisection."""
+    sp = pytest.importorskip("scipy.sparse")
+    dims, vox = (7, 6, 5), (1.0, 0.8, 1.3)
+    g = oracle.geom(dims, vox)
+    V = int(np.prod(dims))
+    rng = np.random.default_rng(14)
+    lors = random_lors(rng, dims, vox, 60)
+    ev = np.array([np.concatenate([a, b]) for a, b in lors], np.float32)
+    rows, cols, vals = [], [], []
+    for i in range(len(ev)):
+        co, ln = oracle.boxclip_path(g, ev[i, :3], ev[i, 3:])
+        rows += [i] * len(co)
+        cols += co.tolist()
+        vals += ln.tolist()
+    A = sp.csr_matrix((vals, (rows, cols)), shape=(len(ev), V))
+    s = oracle.sensitivity(g, ev)
+    np.testing.assert_allclose(s, A.T @ np.ones(len(ev)), rtol=1e-12, atol=1e-13)
+    chords = sum(chord_by_bisection(dims, vox, ev[i, :3].astype(float), ev[i, 3:].astype(float))
+                 for i in range(len(ev)))
+    assert abs(s.sum() - chords) <= 1e-11 * chords

@@ -351,3 +351,41 @@ def test_zslab_passes_match_oracle_c2(pkg):
     rec.close()
     ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev, s, np.ones(cfg.n_voxels))
     assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+# ------------------------------------------------------------------ sensitivity image (NEXT-3)
+@pytest.mark.parametrize("name,n,slabs", [("C1", 10_000, 0), ("C2", 100_000, 0), ("C2", 50_000, 3)])
+def test_sensitivity_matches_oracle(pkg, name, n, slabs):
+    cfg = lmgen.CONFIGS[name]
+    ev = lmgen.events(cfg, 0, n)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(np.ones(cfg.n_voxels, np.float32)))
+    rec.set_slabs(slabs)
+    out = torch.empty(cfg.n_voxels, device="cuda")
+    rec.sensitivity(dev(ev), out)
+    rec.synchronize()
+    got = out.cpu().numpy().astype(np.float64)
+    rec.close()
+    ref = oracle.sensitivity(oracle.geom(cfg.dims, cfg.voxel_mm), ev)
+    assert np.all((got > 0) == (ref > 0))
+    # s enters the update as a divisor: the one-subset bar of north_star applies
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+    assert abs(got.sum() - ref.sum()) <= 1e-6 * ref.sum()
+
+
+def test_set_norm_from_sensitivity(pkg):
+    """A sensitivity computed on the GPU, installed with set_norm, drives the update."""
+    cfg, ev, _ = inputs("C1")
+    ev0 = ev[:cfg.n_events]
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, np.ones(cfg.n_voxels, np.float32))
+    sens = torch.empty(cfg.n_voxels, device="cuda")
+    rec.sensitivity(dev(ev0), sens)
+    rec.set_norm(sens)
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.subset_step(dev(ev0), f)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    rec.close()
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    s_ref = oracle.sensitivity(g, ev0).astype(np.float32)
+    ref = oracle.subset_step(g, ev0, s_ref, np.ones(cfg.n_voxels))
+    assert maxrel(got, ref) <= MAXREL_SUBSET

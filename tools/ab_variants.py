@@ -10,7 +10,8 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 VARIANTS = {
     "default": [],
-    "unfused": ["LMK_FUSED_GATHER=0"],
+    "recompute": ["LMK_RECOMPUTE=1"],
+    "recompute_c256x4": ["LMK_RECOMPUTE=1", "LMK_MIN_BLOCKS=4"],
 }
 
 
