@@ -52,6 +52,7 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-sample", type=int, default=200_000, help="events in the oracle's timed sample")
+    ap.add_argument("--slabs", type=int, default=0, help="z-slab passes for step 1 (0 = automatic)")
     return ap.parse_args()
 
 
@@ -209,6 +210,7 @@ def main():
     flush = torch.empty(FLUSH_BYTES // 4, device=dev)
     stream = torch.cuda.current_stream()
     rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, norm, dist=pkg.make_dist(rank, world), stream=stream)
+    rec.set_slabs(args.slabs)
     N = cfg.n_events
 
     def subset(k):
@@ -316,7 +318,8 @@ def main():
         "config": {"workload": f"{name}: {cfg.note} LM-OSEM {cfg.dims[0]}x{cfg.dims[1]}x{cfg.dims[2]} @ "
                                f"{cfg.voxel_mm[0]} mm, {L} subsets x {N} events, 1 iteration",
                    "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block, f copy, c allreduce)",
-                   "l2": "flushed before every timed step (256 MB write outside the step events)"},
+                   "l2": "flushed before every timed step (256 MB write outside the step events)",
+                   "z_slabs": rec.slabs},
         "s_per_recon": tot_ms / K * L * 1e-3, "s_per_recon_e2e": s_recon,
         "phase_ms_per_step": {"convert_f": conv_ms / K, "project": proj_ms / K, "combine": comb_ms / K,
                               "update": upd_ms / K},

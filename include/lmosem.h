@@ -65,9 +65,10 @@ typedef enum {
 
 #define LMOSEM_NCCL_ID_BYTES 128
 
-/* Multi-GPU setup; pass NULL (or world == 1) for a single GPU. nccl_unique_id points to
+/* Multi-GPU setup; pass NULL for a single GPU without NCCL. nccl_unique_id points to
  * LMOSEM_NCCL_ID_BYTES bytes produced by lmosem_nccl_unique_id on one rank and broadcast
- * to all (the Python binding uses torch.distributed for the broadcast). */
+ * to all (the Python binding uses torch.distributed for the broadcast). A non-NULL dist
+ * always creates the NCCL communicator and runs the combine (world == 1 included). */
 typedef struct {
     int32_t rank, world;
     const void* nccl_unique_id;
@@ -102,7 +103,8 @@ lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
  *   dims[3]     = {nx, ny, nz} > 0, V < 2^31
  *   voxel_mm[3] = voxel size in mm, finite and > 0
  *   norm        = V float32 sensitivity image s (device or host); copied, caller keeps it
- *   dist        = NULL for one GPU, else the rank/world/NCCL id (collective init)
+ *   dist        = NULL for one GPU, else the rank/world/NCCL id (collective init;
+ *                 EINVAL if world < 1, rank outside [0, world) or the id is NULL)
  * Returns EINVAL / ENOMEM / ECUDA / ENCCL; *out is NULL on failure. */
 lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
                           const float* norm, const lmosem_dist* dist);

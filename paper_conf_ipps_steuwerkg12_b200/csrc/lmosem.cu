@@ -225,7 +225,7 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
     if ((s = mark(ctx, pm, 1))) return s;
     if ((s = launch_project(ctx, ev + b, e - b, nullptr, 0))) return s;
     if ((s = mark(ctx, pm, 2))) return s;
-    if (ctx->world > 1) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    if (ctx->comm) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
     if ((s = mark(ctx, pm, 3))) return s;
     if ((s = launch_update(ctx, write_f ? f : nullptr))) return s;
     if ((s = mark(ctx, pm, 4))) return s;
@@ -302,7 +302,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         rank = dist->rank;
         world = dist->world;
         if (world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
-        if (world > 1 && !dist->nccl_unique_id) return LMOSEM_EINVAL;
+        if (!dist->nccl_unique_id) return LMOSEM_EINVAL;
     }
     lmosem_ctx* ctx = new (std::nothrow) lmosem_ctx;
     if (!ctx) return LMOSEM_ENOMEM;
@@ -403,7 +403,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
     cuda(cudaStreamSynchronize(ctx->stream), "sync");
     if (s != LMOSEM_OK) return bail(s);
-    if (world > 1) {
+    if (dist) {  // a communicator whenever a dist is given (world == 1 runs the 1-rank all-reduce)
         ncclUniqueId id;
         std::memcpy(&id, dist->nccl_unique_id, sizeof(id));
         ncclResult_t r = ncclCommInitRank(&ctx->comm, world, id, rank);
@@ -550,7 +550,7 @@ LMOSEM_API lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event*
     block_range(n_events, ctx->rank, ctx->world, &b, &e);
     lmosem_status s;
     if ((s = launch_project(ctx, events + b, e - b, nullptr, 4))) return s;
-    if (ctx->world > 1) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    if (ctx->comm) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
     return launch_to_row(ctx, ctx->c, s_out, 1);  // s_out <- c, c <- 0
 }
 
@@ -576,7 +576,7 @@ LMOSEM_API lmosem_status lmosem_synchronize(lmosem_ctx* ctx) {
     USABLE(ctx);
     CK(cudaStreamSynchronize(ctx->stream));
     CK(cudaStreamSynchronize(ctx->copy_stream));
-    if (ctx->world > 1 && ctx->comm) {
+    if (ctx->comm) {
         ncclResult_t async_err = ncclSuccess;
         NK(ncclCommGetAsyncError(ctx->comm, &async_err));
         if (async_err != ncclSuccess)

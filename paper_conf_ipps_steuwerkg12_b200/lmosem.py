@@ -287,7 +287,7 @@ class Reconstructor:
 
 
 def make_dist(rank: int, world: int, group=None) -> tuple[int, int, bytes] | None:
-    """NCCL id from rank 0, broadcast with torch.distributed (any backend)."""
+    """NCCL id from rank 0, broadcast with torch.distributed (any backend). None for world 1."""
     if world <= 1:
         return None
     import torch.distributed as dist

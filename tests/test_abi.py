@@ -83,7 +83,7 @@ def test_init_einval_pointers_and_dist(lib):
     assert lib.lmosem_init(None, d, v, 1, None) == L.EINVAL
     assert lib.lmosem_init(ctypes.byref(h), None, v, 1, None) == L.EINVAL
     assert lib.lmosem_init(ctypes.byref(h), d, v, None, None) == L.EINVAL
-    for rank, world, uid in [(0, 0, 1), (2, 2, 1), (-1, 2, 1), (0, 2, None)]:
+    for rank, world, uid in [(0, 0, 1), (2, 2, 1), (-1, 2, 1), (0, 2, None), (0, 1, None)]:
         dist = L.Dist(rank, world, uid)
         assert lib.lmosem_init(ctypes.byref(h), d, v, 1, ctypes.byref(dist)) == L.EINVAL
 

@@ -389,3 +389,21 @@ def test_set_norm_from_sensitivity(pkg):
     s_ref = oracle.sensitivity(g, ev0).astype(np.float32)
     ref = oracle.subset_step(g, ev0, s_ref, np.ones(cfg.n_voxels))
     assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+def test_nccl_combine_single_rank(pkg):
+    """The NCCL path (communicator from a broadcast id, in-place all-reduce of c on the
+    compute stream) on the one GPU available: a 1-rank context must match the plain one."""
+    cfg, ev, s = inputs("C1")
+    ev0 = dev(ev[:cfg.n_events])
+    rec0 = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    rec1 = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), dist=(0, 1, pkg.nccl_unique_id()))
+    f0 = dev(np.ones(cfg.n_voxels, np.float32))
+    f1 = dev(np.ones(cfg.n_voxels, np.float32))
+    rec0.subset_step(ev0, f0)
+    rec1.subset_step(ev0, f1)
+    rec0.synchronize()
+    rec1.synchronize()
+    torch.testing.assert_close(f1, f0, rtol=1e-6, atol=0)
+    rec0.close()
+    rec1.close()
