@@ -10,8 +10,7 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 VARIANTS = {
     "default": [],
-    "recompute": ["LMK_RECOMPUTE=1"],
-    "recompute_c256x4": ["LMK_RECOMPUTE=1", "LMK_MIN_BLOCKS=4"],
+    "path_gather": ["LMK_PATH_GATHER=1"],
 }
 
 
