@@ -50,16 +50,22 @@ __device__ __forceinline__ int bidx(int A, int B, int p) { return A * p + B * (p
 // (<= 2^-41 per slab) accumulates to < 1e-9 voxel over 600 slabs.
 constexpr int FIX_BITS = 40;
 
-// Per-LOR traversal state (broadcast lane -> warp by shuffles).
+// Per-LOR traversal state (broadcast lane -> warp by shuffles; 16 registers).
 struct Lor {
     long long wb0, wc0;  // minor-axis positions at the plane u_a = i0 (Q24.40 voxels)
     long long sb, sc;    // du_b/du_a, du_c/du_a (Q24.40)
-    float ab, bb, ac, bc;  // crossing offset in a slab: d = fma(g, a, b) (+inf if no step)
+    float ab, ac;     // crossing offset in a slab: d = g * a (g: distance to the plane, Q.40)
     float lunit;      // mm of chord per unit of u_a
     float fin, fout;  // clip inside the first / last slab (local coordinate in [0,1])
     int i0, ns;       // first slab index along a, number of slabs
+    int code;         // bits 0-1: dominant axis a; 2-3: step of b (1: +1, 3: -1, 0: none); 4-5: c
+};
+
+// Warp-uniform constants derived from Lor::code and the grid once per LOR.
+struct Walk {
+    int stb, stc;     // minor-axis steps (+1, -1, 0)
+    float bb, bc;     // 0, or +inf for an axis without a step (no crossing)
     int Aa, Ba, Ab, Bb, Ac, Bc;  // brick index coefficients of axes a, b, c
-    int steps;        // bits 0-1: step of b (+1 -> 1, -1 -> 3, 0 -> 0); bits 2-3: same for c
 };
 
 template <class T>
@@ -120,18 +126,13 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     // of travel, divided by |slope|: d = g * 2^-40 / |s| (no step: never, d = +inf)
     const float isb = (float)(1.0 / (fabs(sb) * fx)), isc = (float)(1.0 / (fabs(sc) * fx));
     L.ab = sb != 0.0 ? isb : 0.0f;
-    L.bb = sb != 0.0 ? 0.0f : CUDART_INF_F;
     L.ac = sc != 0.0 ? isc : 0.0f;
-    L.bc = sc != 0.0 ? 0.0f : CUDART_INF_F;
     L.lunit = (float)(Lmm * fabs(rDa));
     L.fin = fminf(fmaxf((float)(ua_in - (double)i0), 0.0f), 1.0f);
     L.fout = fminf(fmaxf((float)(ua_out - (double)il), 0.0f), 1.0f);
     L.i0 = i0;
     L.ns = il - i0 + 1;
-    L.Aa = sel3(g.A, a); L.Ba = sel3(g.B, a);
-    L.Ab = sel3(g.A, b); L.Bb = sel3(g.B, b);
-    L.Ac = sel3(g.A, c); L.Bc = sel3(g.B, c);
-    L.steps = (sb > 0.0 ? 1 : (sb < 0.0 ? 3 : 0)) | (sc > 0.0 ? 4 : (sc < 0.0 ? 12 : 0));
+    L.code = a | (sb > 0.0 ? 4 : (sb < 0.0 ? 12 : 0)) | (sc > 0.0 ? 16 : (sc < 0.0 ? 48 : 0));
     return true;
 }
 
@@ -166,22 +167,28 @@ __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     L.sb = shfl_ll(s.sb, src);
     L.sc = shfl_ll(s.sc, src);
     L.ab = __shfl_sync(0xffffffffu, s.ab, src);
-    L.bb = __shfl_sync(0xffffffffu, s.bb, src);
     L.ac = __shfl_sync(0xffffffffu, s.ac, src);
-    L.bc = __shfl_sync(0xffffffffu, s.bc, src);
     L.lunit = __shfl_sync(0xffffffffu, s.lunit, src);
     L.fin = __shfl_sync(0xffffffffu, s.fin, src);
     L.fout = __shfl_sync(0xffffffffu, s.fout, src);
     L.i0 = __shfl_sync(0xffffffffu, s.i0, src);
     L.ns = __shfl_sync(0xffffffffu, s.ns, src);
-    L.Aa = __shfl_sync(0xffffffffu, s.Aa, src);
-    L.Ba = __shfl_sync(0xffffffffu, s.Ba, src);
-    L.Ab = __shfl_sync(0xffffffffu, s.Ab, src);
-    L.Bb = __shfl_sync(0xffffffffu, s.Bb, src);
-    L.Ac = __shfl_sync(0xffffffffu, s.Ac, src);
-    L.Bc = __shfl_sync(0xffffffffu, s.Bc, src);
-    L.steps = __shfl_sync(0xffffffffu, s.steps, src);
+    L.code = __shfl_sync(0xffffffffu, s.code, src);
     return L;
+}
+
+__device__ __forceinline__ Walk make_walk(const Lor& L, const GridGeom& g) {
+    Walk W;
+    const int a = L.code & 3, b = (a == 0) ? 1 : 0, c = (a == 2) ? 1 : 2;
+    const int cb = (L.code >> 2) & 3, cc = (L.code >> 4) & 3;
+    W.stb = (cb == 1) - (cb == 3);
+    W.stc = (cc == 1) - (cc == 3);
+    W.bb = cb ? 0.0f : CUDART_INF_F;
+    W.bc = cc ? 0.0f : CUDART_INF_F;
+    W.Aa = sel3(g.A, a); W.Ba = sel3(g.B, a);
+    W.Ab = sel3(g.A, b); W.Bb = sel3(g.B, b);
+    W.Ac = sel3(g.A, c); W.Bc = sel3(g.B, c);
+    return W;
 }
 
 // The (up to) three pieces of slab k: j = brick index, l = chord length in mm (0 for
@@ -191,19 +198,22 @@ struct Pieces {
     float l0, l1, l2;
 };
 
-__device__ __forceinline__ Pieces slab_pieces(const Lor& L, int k, int stb, int stc) {
+// Slab k of the LOR; wb, wc = minor positions at its plane (Q24.40), Ja = brick index
+// contribution of its dominant-axis coordinate (the caller steps all three exactly).
+__device__ __forceinline__ Pieces slab_pieces(const Lor& L, const Walk& W, int k, long long wb, long long wc,
+                                              int Ja) {
+    const int stb = W.stb, stc = W.stc;
     int ib, ic;
-    const float gb = fix_to_plane(L.wb0 + (long long)k * L.sb, stb > 0, ib);
-    const float gc = fix_to_plane(L.wc0 + (long long)k * L.sc, stc > 0, ic);
-    const float db = fmaf(gb, L.ab, L.bb);  // crossing offsets along u_a in the slab
-    const float dc = fmaf(gc, L.ac, L.bc);
+    const float gb = fix_to_plane(wb, stb > 0, ib);
+    const float gc = fix_to_plane(wc, stc > 0, ic);
+    const float db = fmaf(gb, L.ab, W.bb);  // crossing offsets along u_a in the slab
+    const float dc = fmaf(gc, L.ac, W.bc);
     const float dlo = (k == 0) ? L.fin : 0.0f;
     const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;
     const float q1 = fminf(fmaxf(fminf(db, dc), dlo), dhi);
     const float q2 = fminf(fmaxf(fmaxf(db, dc), dlo), dhi);
-    const int Ja = bidx(L.Aa, L.Ba, L.i0 + k + HALO_LO);
-    const int Jb0 = bidx(L.Ab, L.Bb, ib + HALO_LO), Jb1 = bidx(L.Ab, L.Bb, ib + HALO_LO + stb);
-    const int Jc0 = bidx(L.Ac, L.Bc, ic + HALO_LO), Jc1 = bidx(L.Ac, L.Bc, ic + HALO_LO + stc);
+    const int Jb0 = bidx(W.Ab, W.Bb, ib + HALO_LO), Jb1 = bidx(W.Ab, W.Bb, ib + HALO_LO + stb);
+    const int Jc0 = bidx(W.Ac, W.Bc, ic + HALO_LO), Jc1 = bidx(W.Ac, W.Bc, ic + HALO_LO + stc);
     // piece 0 before both crossings, piece 2 after both, piece 1 after the first one
     Pieces P;
     P.j0 = Ja + Jb0 + Jc0;
@@ -213,6 +223,30 @@ __device__ __forceinline__ Pieces slab_pieces(const Lor& L, int k, int stb, int 
     P.l1 = (q2 - q1) * L.lunit;
     P.l2 = (dhi - q2) * L.lunit;
     return P;
+}
+
+// Per-lane stepping state of a LOR's geometry loop: lane l visits slabs l, l+32, ...;
+// positions advance by exactly 32 slopes (integer adds), so w(k) = w0 + k*s exactly.
+struct Step {
+    long long wb, wc, dwb, dwc;
+    int Ja, dJa;
+};
+
+__device__ __forceinline__ Step make_step(const Lor& L, const Walk& W, int lane) {
+    Step S;
+    S.wb = L.wb0 + (long long)lane * L.sb;
+    S.wc = L.wc0 + (long long)lane * L.sc;
+    S.dwb = 32LL * L.sb;
+    S.dwc = 32LL * L.sc;
+    S.Ja = bidx(W.Aa, W.Ba, L.i0 + lane + HALO_LO);  // 32 slabs later: same parity
+    S.dJa = 32 * W.Aa;
+    return S;
+}
+
+__device__ __forceinline__ void advance(Step& S) {
+    S.wb += S.dwb;
+    S.wc += S.dwc;
+    S.Ja += S.dJa;
 }
 
 __device__ __forceinline__ float warp_sum(float v) {
@@ -232,14 +266,26 @@ __device__ __forceinline__ void load_event(const float* __restrict__ events, int
 // Appends the valid pieces of every lane to the warp's path buffer in path order
 // (lane-major = slab order, then piece order): the exclusive prefix of the per-lane
 // counts n = v0 + v1 + v2 (0..3) comes from two ballots on its bits.
-__device__ __forceinline__ void append3(int2* __restrict__ path, int& cnt, unsigned lt, const Pieces& P, bool v0,
-                                        bool v1, bool v2) {
-    const int n = (int)v0 + (int)v1 + (int)v2;
-    const unsigned b0 = __ballot_sync(0xffffffffu, n & 1), b1 = __ballot_sync(0xffffffffu, n & 2);
-    const int pos = cnt + __popc(b0 & lt) + 2 * __popc(b1 & lt);
-    if (v0) path[pos] = make_int2(P.j0, __float_as_int(P.l0));
-    if (v1) path[pos + v0] = make_int2(P.j1, __float_as_int(P.l1));
-    if (v2) path[pos + v0 + v1] = make_int2(P.j2, __float_as_int(P.l2));
+__device__ __forceinline__ void sts2(unsigned addr, int j, float l) {
+    asm volatile("st.shared.v2.b32 [%0], {%1, %2};" ::"r"(addr), "r"(j), "r"(__float_as_int(l)) : "memory");
+}
+
+__device__ __forceinline__ int2 lds2(unsigned addr) {
+    int2 v;
+    asm volatile("ld.shared.v2.b32 {%0, %1}, [%2];" : "=r"(v.x), "=r"(v.y) : "r"(addr) : "memory");
+    return v;
+}
+
+// path_s: 32-bit shared-window address of the warp's path buffer (8 B per piece).
+__device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, const Pieces& P, bool v0, bool v1,
+                                        bool v2) {
+    // n = v0 + v1 + v2: bit 0 = parity, bit 1 = majority
+    const unsigned b0 = __ballot_sync(0xffffffffu, v0 ^ v1 ^ v2);
+    const unsigned b1 = __ballot_sync(0xffffffffu, (v0 & v1) | (v0 & v2) | (v1 & v2));
+    const unsigned a = path_s + 8u * (unsigned)(cnt + __popc(b0 & lt) + 2 * __popc(b1 & lt));
+    if (v0) sts2(a, P.j0, P.l0);
+    if (v1) sts2(a + 8u * v0, P.j1, P.l1);
+    if (v2) sts2(a + 8u * (v0 + v1), P.j2, P.l2);
     cnt += __popc(b0) + 2 * __popc(b1);
 }
 
@@ -274,7 +320,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
-    int2* path = smem_path + (size_t)wib * cap;
+    const unsigned path_s = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)wib * cap);
     const unsigned lt = (1u << lane) - 1u;
     const int64_t warp = (int64_t)blockIdx.x * (blockDim.x >> 5) + wib;
     const int64_t nwarps = (int64_t)gridDim.x * (blockDim.x >> 5);
@@ -298,20 +344,20 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
             const int src = __ffs(mask) - 1;
             mask &= mask - 1;
             const Lor L = shfl_lor(mine, src);
-            const int stb = ((L.steps & 3) == 1) - ((L.steps & 3) == 3);
-            const int stc = ((L.steps & 12) == 4) - ((L.steps & 12) == 12);
-            // pass 1: geometry (uniform loop: lanes past the last slab recompute it and drop
-            // their pieces) -> path pieces in shared memory (when back-projecting) and f
+            const Walk W = make_walk(L, g);
+            // pass 1: geometry (uniform loop; lanes past the last slab drop their pieces) -> path pieces in shared memory (when back-projecting) and f
             // gathered in the same loop (when forward-projecting): each iteration consumes
             // the previous iteration's loads, so their latency overlaps the next batch
             int cnt = 0;
             float acc = 0.0f;
             float g0 = 0.f, g1 = 0.f, g2 = 0.f, w0 = 0.f, w1 = 0.f, w2 = 0.f;
-            for (int k0 = 0; k0 < L.ns; k0 += 32) {
-                const bool in = k0 + lane < L.ns;
-                const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
+            Step S = make_step(L, W, lane);
+            for (int k0 = 0; k0 < L.ns; k0 += 32, advance(S)) {
+                const int k = k0 + lane;
+                const bool in = k < L.ns;  // lanes past the last slab compute garbage, store nothing
+                const Pieces P = slab_pieces(L, W, k, S.wb, S.wc, S.Ja);
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
-                if (kStore) append3(path, cnt, lt, P, v0, v1, v2);
+                if (kStore) append3(path_s, cnt, lt, P, v0, v1, v2);
                 if (kGather) {
                     acc = fmaf(g0, w0, acc);
                     acc = fmaf(g1, w1, acc);
@@ -341,13 +387,14 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 if (kStore) {
 #pragma unroll 8
                     for (int m = lane; m < cnt; m += 32) {
-                        const int2 q = path[m];
+                        const int2 q = lds2(path_s + 8u * (unsigned)m);
                         atomicAdd(cb + q.x, __int_as_float(q.y) * inv);
                     }
                 } else {
-                    for (int k0 = 0; k0 < L.ns; k0 += 32) {
+                    Step S = make_step(L, W, lane);
+                    for (int k0 = 0; k0 < L.ns; k0 += 32, advance(S)) {
                         const bool in = k0 + lane < L.ns;
-                        const Pieces P = slab_pieces(L, in ? k0 + lane : L.ns - 1, stb, stc);
+                        const Pieces P = slab_pieces(L, W, k0 + lane, S.wb, S.wc, S.Ja);
                         if (in && P.l0 > 0.0f) atomicAdd(cb + P.j0, P.l0 * inv);
                         if (in && P.l1 > 0.0f) atomicAdd(cb + P.j1, P.l1 * inv);
                         if (in && P.l2 > 0.0f) atomicAdd(cb + P.j2, P.l2 * inv);

@@ -10,7 +10,8 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 VARIANTS = {
     "default": [],
-    "path_gather": ["LMK_PATH_GATHER=1"],
+    "c256x2": ["LMK_MIN_BLOCKS=2"],
+    "c128x5": ["LMK_CTA_THREADS=128", "LMK_MIN_BLOCKS=5"],
 }
 
 
