@@ -52,8 +52,8 @@ constexpr int FIX_BITS = 40;
 
 // Per-LOR traversal state (broadcast lane -> warp by shuffles; 16 registers).
 struct Lor {
-    long long wb0, wc0;  // minor-axis positions at the plane u_a = i0 (Q24.40 voxels)
-    long long sb, sc;    // du_b/du_a, du_c/du_a (Q24.40)
+    long long wb0, wc0;  // minor-axis positions at the plane u_a = i0 (Q24.40 voxels, stored frame)
+    long long sb, sc;    // their change per slab (stored frame: <= 0)
     float ab, ac;     // crossing offset in a slab: d = g * a (g: distance to the plane, Q.40)
     float lunit;      // mm of chord per unit of u_a
     float fin, fout;  // clip inside the first / last slab (local coordinate in [0,1])
@@ -63,9 +63,10 @@ struct Lor {
 
 // Warp-uniform constants derived from Lor::code and the grid once per LOR.
 struct Walk {
-    int stb, stc;     // minor-axis steps (+1, -1, 0)
+    int mb, mc;       // -1 for a mirrored (up-moving) axis, else 0: voxel index = floor(w) ^ m
     float bb, bc;     // 0, or +inf for an axis without a step (no crossing)
     int Aa, Ba, Ab, Bb, Ac, Bc;  // brick index coefficients of axes a, b, c
+    int Db0, Db1, Dc0, Dc1;      // index change of a step for an even / odd padded coordinate
 };
 
 template <class T>
@@ -118,10 +119,18 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     const double rDa = 1.0 / Da;
     const double sb = Db * rDa, sc = Dc * rDa;
     const double fx = (double)(1LL << FIX_BITS);
-    L.sb = __double2ll_rn(sb * fx);
-    L.sc = __double2ll_rn(sc * fx);
-    L.wb0 = __double2ll_rn((u1b + ((double)i0 - u1a) * sb) * fx);
-    L.wc0 = __double2ll_rn((u1c + ((double)i0 - u1a) * sc) * fx);
+    // stored frame: an axis moving up is mirrored, w' = -w - 2^-40, so every moving axis
+    // moves down and its distance to the next plane is its fraction (the 2^-40 offset keeps
+    // an exactly integral position inside its half-open voxel: distance = one voxel)
+    {
+        const long long wb = __double2ll_rn((u1b + ((double)i0 - u1a) * sb) * fx);
+        const long long wc = __double2ll_rn((u1c + ((double)i0 - u1a) * sc) * fx);
+        const long long qb = __double2ll_rn(sb * fx), qc = __double2ll_rn(sc * fx);
+        L.wb0 = sb > 0.0 ? -wb - 1 : wb;
+        L.sb = sb > 0.0 ? -qb : qb;
+        L.wc0 = sc > 0.0 ? -wc - 1 : wc;
+        L.sc = sc > 0.0 ? -qc : qc;
+    }
     // crossing inside a slab: distance g (Q.40 units) to the next plane in the direction
     // of travel, divided by |slope|: d = g * 2^-40 / |s| (no step: never, d = +inf)
     const float isb = (float)(1.0 / (fabs(sb) * fx)), isc = (float)(1.0 / (fabs(sc) * fx));
@@ -150,16 +159,6 @@ __device__ __forceinline__ long long shfl_ll(long long v, int src) {
     return (long long)(((unsigned long long)(unsigned)hi << 32) | (unsigned)lo);
 }
 
-// Q24.40 position w -> floor (int) and the exact distance to the next voxel plane in
-// the direction of travel (up: 2^40 - frac, down: frac), converted to float with full
-// relative precision (the crossing offset divides it by |slope|, so an absolute
-// rounding error here would be amplified for shallow minor axes).
-__device__ __forceinline__ float fix_to_plane(long long w, bool up, int& fl) {
-    fl = (int)(w >> FIX_BITS);
-    const unsigned long long frac = (unsigned long long)w & ((1ULL << FIX_BITS) - 1ULL);
-    return __ull2float_rn(up ? (1ULL << FIX_BITS) - frac : frac);
-}
-
 __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     Lor L;
     L.wb0 = shfl_ll(s.wb0, src);
@@ -181,13 +180,19 @@ __device__ __forceinline__ Walk make_walk(const Lor& L, const GridGeom& g) {
     Walk W;
     const int a = L.code & 3, b = (a == 0) ? 1 : 0, c = (a == 2) ? 1 : 2;
     const int cb = (L.code >> 2) & 3, cc = (L.code >> 4) & 3;
-    W.stb = (cb == 1) - (cb == 3);
-    W.stc = (cc == 1) - (cc == 3);
+    const int stb = (cb == 1) - (cb == 3), stc = (cc == 1) - (cc == 3);
+    W.mb = -(stb > 0);
+    W.mc = -(stc > 0);
     W.bb = cb ? 0.0f : CUDART_INF_F;
     W.bc = cc ? 0.0f : CUDART_INF_F;
     W.Aa = sel3(g.A, a); W.Ba = sel3(g.B, a);
     W.Ab = sel3(g.A, b); W.Bb = sel3(g.B, b);
     W.Ac = sel3(g.A, c); W.Bc = sel3(g.B, c);
+    // J(p + st) - J(p) = st*A + B*((p + st)&1 - (p&1)) = st*A + B (p even), st*A - B (p odd)
+    W.Db0 = stb ? stb * W.Ab + W.Bb : 0;
+    W.Db1 = stb ? stb * W.Ab - W.Bb : 0;
+    W.Dc0 = stc ? stc * W.Ac + W.Bc : 0;
+    W.Dc1 = stc ? stc * W.Ac - W.Bc : 0;
     return W;
 }
 
@@ -200,20 +205,37 @@ struct Pieces {
 
 // Slab k of the LOR; wb, wc = minor positions at its plane (Q24.40), Ja = brick index
 // contribution of its dominant-axis coordinate (the caller steps all three exactly).
+// floor (int) and fraction (float, exact conversion of the 40 fraction bits) of a
+// stored-frame Q24.40 position; the fraction is the distance to the next plane crossed.
+__device__ __forceinline__ float fix_split(long long w, int& fl) {
+    const unsigned hi = (unsigned)((unsigned long long)w >> 32), lo = (unsigned)w;
+    fl = (int)hi >> (FIX_BITS - 32);
+    return __ull2float_rn(((unsigned long long)(hi & ((1u << (FIX_BITS - 32)) - 1u)) << 32) | lo);
+}
+
+// Brick index of padded coordinate p on one axis (A*p + B*(p&1)) and of p + step.
+__device__ __forceinline__ void bidx2(int A, int B, int D0, int D1, int p, int& J0, int& J1) {
+    const bool odd = p & 1;
+    J0 = A * p + (odd ? B : 0);
+    J1 = J0 + (odd ? D1 : D0);
+}
+
+// Slab k of the LOR; wb, wc = stored-frame minor positions at its plane, Ja = brick
+// index contribution of its dominant-axis coordinate (the caller steps all three).
 __device__ __forceinline__ Pieces slab_pieces(const Lor& L, const Walk& W, int k, long long wb, long long wc,
                                               int Ja) {
-    const int stb = W.stb, stc = W.stc;
-    int ib, ic;
-    const float gb = fix_to_plane(wb, stb > 0, ib);
-    const float gc = fix_to_plane(wc, stc > 0, ic);
+    int fb, fc;
+    const float gb = fix_split(wb, fb), gc = fix_split(wc, fc);
+    const int ib = fb ^ W.mb, ic = fc ^ W.mc;  // voxel indices (un-mirrored)
     const float db = fmaf(gb, L.ab, W.bb);  // crossing offsets along u_a in the slab
     const float dc = fmaf(gc, L.ac, W.bc);
     const float dlo = (k == 0) ? L.fin : 0.0f;
     const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;
     const float q1 = fminf(fmaxf(fminf(db, dc), dlo), dhi);
     const float q2 = fminf(fmaxf(fmaxf(db, dc), dlo), dhi);
-    const int Jb0 = bidx(W.Ab, W.Bb, ib + HALO_LO), Jb1 = bidx(W.Ab, W.Bb, ib + HALO_LO + stb);
-    const int Jc0 = bidx(W.Ac, W.Bc, ic + HALO_LO), Jc1 = bidx(W.Ac, W.Bc, ic + HALO_LO + stc);
+    int Jb0, Jb1, Jc0, Jc1;
+    bidx2(W.Ab, W.Bb, W.Db0, W.Db1, ib, Jb0, Jb1);  // halo offsets of b, c are in Ja
+    bidx2(W.Ac, W.Bc, W.Dc0, W.Dc1, ic, Jc0, Jc1);
     // piece 0 before both crossings, piece 2 after both, piece 1 after the first one
     Pieces P;
     P.j0 = Ja + Jb0 + Jc0;
@@ -238,7 +260,9 @@ __device__ __forceinline__ Step make_step(const Lor& L, const Walk& W, int lane)
     S.wc = L.wc0 + (long long)lane * L.sc;
     S.dwb = 32LL * L.sb;
     S.dwc = 32LL * L.sc;
-    S.Ja = bidx(W.Aa, W.Ba, L.i0 + lane + HALO_LO);  // 32 slabs later: same parity
+    // 32 slabs later: same parity. HALO_LO is even, so J(i + HALO_LO) = J(i) + HALO_LO*A on
+    // every axis: the minor axes' halo offsets are folded in here.
+    S.Ja = bidx(W.Aa, W.Ba, L.i0 + lane + HALO_LO) + HALO_LO * (W.Ab + W.Ac);
     S.dJa = 32 * W.Aa;
     return S;
 }
@@ -279,14 +303,14 @@ __device__ __forceinline__ int2 lds2(unsigned addr) {
 // path_s: 32-bit shared-window address of the warp's path buffer (8 B per piece).
 __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, const Pieces& P, bool v0, bool v1,
                                         bool v2) {
-    // n = v0 + v1 + v2: bit 0 = parity, bit 1 = majority
-    const unsigned b0 = __ballot_sync(0xffffffffu, v0 ^ v1 ^ v2);
-    const unsigned b1 = __ballot_sync(0xffffffffu, (v0 & v1) | (v0 & v2) | (v1 & v2));
-    const unsigned a = path_s + 8u * (unsigned)(cnt + __popc(b0 & lt) + 2 * __popc(b1 & lt));
+    // exclusive prefix over lanes of v0 + v1 + v2 from three predicate ballots
+    const unsigned b0 = __ballot_sync(0xffffffffu, v0), b1 = __ballot_sync(0xffffffffu, v1),
+                   b2 = __ballot_sync(0xffffffffu, v2);
+    const unsigned a = path_s + 8u * (unsigned)(cnt + __popc(b0 & lt) + __popc(b1 & lt) + __popc(b2 & lt));
     if (v0) sts2(a, P.j0, P.l0);
-    if (v1) sts2(a + 8u * v0, P.j1, P.l1);
-    if (v2) sts2(a + 8u * (v0 + v1), P.j2, P.l2);
-    cnt += __popc(b0) + 2 * __popc(b1);
+    if (v1) sts2(a + (v0 ? 8u : 0u), P.j1, P.l1);
+    if (v2) sts2(a + (v0 ? 8u : 0u) + (v1 ? 8u : 0u), P.j2, P.l2);
+    cnt += __popc(b0) + __popc(b1) + __popc(b2);
 }
 
 #ifndef LMK_CTA_THREADS
@@ -345,12 +369,11 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
             mask &= mask - 1;
             const Lor L = shfl_lor(mine, src);
             const Walk W = make_walk(L, g);
-            // pass 1: geometry (uniform loop; lanes past the last slab drop their pieces) -> path pieces in shared memory (when back-projecting) and f
-            // gathered in the same loop (when forward-projecting): each iteration consumes
-            // the previous iteration's loads, so their latency overlaps the next batch
+            // pass 1: geometry (uniform loop; lanes past the last slab drop their pieces)
+            // -> path pieces in shared memory (when back-projecting) and f gathered in the
+            // same loop (when forward-projecting)
             int cnt = 0;
             float acc = 0.0f;
-            float g0 = 0.f, g1 = 0.f, g2 = 0.f, w0 = 0.f, w1 = 0.f, w2 = 0.f;
             Step S = make_step(L, W, lane);
             for (int k0 = 0; k0 < L.ns; k0 += 32, advance(S)) {
                 const int k = k0 + lane;
@@ -359,20 +382,13 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
                 if (kStore) append3(path_s, cnt, lt, P, v0, v1, v2);
                 if (kGather) {
-                    acc = fmaf(g0, w0, acc);
-                    acc = fmaf(g1, w1, acc);
-                    acc = fmaf(g2, w2, acc);
-                    g0 = v0 ? __ldg(fb + P.j0) : 0.f;
-                    g1 = v1 ? __ldg(fb + P.j1) : 0.f;
-                    g2 = v2 ? __ldg(fb + P.j2) : 0.f;
-                    w0 = P.l0; w1 = P.l1; w2 = P.l2;
+                    acc = fmaf(v0 ? __ldg(fb + P.j0) : 0.f, P.l0, acc);
+                    acc = fmaf(v1 ? __ldg(fb + P.j1) : 0.f, P.l1, acc);
+                    acc = fmaf(v2 ? __ldg(fb + P.j2) : 0.f, P.l2, acc);
                 }
             }
             float fpv = fp_known;
             if (kGather) {
-                acc = fmaf(g0, w0, acc);
-                acc = fmaf(g1, w1, acc);
-                acc = fmaf(g2, w2, acc);
                 fpv = warp_sum(acc);
                 if (MODE == 1 && lane == 0) fp[base + src] = fpv;
                 if (MODE == 2 && lane == 0) fp[base + src] += fpv;

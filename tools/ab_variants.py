@@ -10,8 +10,7 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 VARIANTS = {
     "default": [],
-    "c256x2": ["LMK_MIN_BLOCKS=2"],
-    "c128x5": ["LMK_CTA_THREADS=128", "LMK_MIN_BLOCKS=5"],
+    "nopipe": ["LMK_PIPE_GATHER=0"],
 }
 
 
