@@ -291,8 +291,18 @@ def main():
     proj_avg_s = proj_ms / K * 1e-3
     l2 = l2_peak_gbs(cfg.n_voxels)
     alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0  # 4 B gather + 4 B RED per path element, 24 B/event
+    traffic = None
+    try:
+        with open(os.path.join(ROOT, "profiles", "r01_traffic.json")) as fh:
+            t = json.load(fh).get(name)
+        if t:
+            traffic = t["dram_bytes_read_per_launch"] + t["dram_bytes_write_per_launch"]
+    except (OSError, ValueError, KeyError):
+        pass
     roof = {"kernel": "k_project<0> (fused Siddon + forward + back-projection)", "bound": "l2",
-            "achieved": alg_l2_bytes / proj_avg_s / 1e9, "unit": "GB/s", "traffic": None,
+            "achieved": alg_l2_bytes / proj_avg_s / 1e9, "unit": "GB/s", "traffic": traffic,
+            "traffic_note": "DRAM bytes per launch (ncu --set full, profiles/r01_traffic.json); the algorithmic "
+                            "bytes are L2 traffic, the images stay L2-resident",
             "per_unit": f"{mean_path} path elements x (4 B f gather + 4 B c RED) + 24 B event per event",
             "units_per_launch": ev_per_launch}
     if l2:
