@@ -257,7 +257,7 @@ def main():
     if not args.no_e2e:
         pinned = torch.from_numpy(ev_host).pin_memory()
         offs = np.arange(L + 1, dtype=np.int64) * N
-        fh = np.ones(cfg.n_voxels, np.float32)
+        fh = torch.ones(cfg.n_voxels, dtype=torch.float32).pin_memory()  # pinned host image
         rec.reconstruct_host(pinned, offs[:2], 1, fh)  # warm-up (allocates the streaming buffers)
         reps = max(1, K // L)
         if world > 1:
@@ -273,7 +273,7 @@ def main():
                "h2d_bytes_per_step": int(24 * (e - b) + 4 * cfg.n_voxels / L),
                "d2h_bytes_per_step": int(4 * cfg.n_voxels / L),
                "note": f"lmosem_reconstruct_host over {L} subsets x {reps} (pinned host events streamed per subset, "
-                       f"overlapped with projection; f H2D/D2H once per reconstruction), wall clock"}
+                       f"overlapped with projection; pinned f H2D/D2H once per reconstruction), wall clock"}
         s_recon = float(te.item()) / reps
     else:
         s_recon = None

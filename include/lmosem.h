@@ -30,9 +30,10 @@
  *  - Distribution (§III.A; §IV.A): with
  *    world > 1, subset_step / reconstruct are collective. Every rank passes the WHOLE
  *    subset; rank r projects the block [floor(r*N/P), floor((r+1)*N/P)) (block
- *    distribution), f is replicated (copy distribution) and c is combined by an NCCL
- *    all-reduce(sum) (copy(add)). Every rank then applies step 2 to its full replica,
- *    so the replicas stay identical.
+ *    distribution), f is replicated (copy distribution) and c is combined by NCCL
+ *    (copy(add)): by default reduce-scatter + block update + all-gather (the paper's
+ *    PSD -> ISD switch), or all-reduce + full update (lmosem_set_combine). Either way the
+ *    replicas of f are identical on return.
  *  - Errors: every call returns a status. EINVAL for bad arguments (nothing enqueued);
  *    ECUDA/ENCCL for runtime failures (message in lmosem_last_error), after which the
  *    context answers ESTATE to everything except lmosem_last_error and lmosem_destroy.
@@ -108,6 +109,20 @@ lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
  * Returns EINVAL / ENOMEM / ECUDA / ENCCL; *out is NULL on failure. */
 lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
                           const float* norm, const lmosem_dist* dist);
+
+/* Combine of the per-GPU error images (world > 1; needs a context created with a dist):
+ *   LMOSEM_COMBINE_ALLREDUCE: ncclAllReduce(c), then every rank updates its full replica;
+ *   LMOSEM_COMBINE_ISD: the paper's PSD -> ISD switch (Listing 3
+ *     l.15-19): ncclReduceScatter(c) gives rank r the sum over its contiguous block of the
+ *     internal image, rank r updates only that block (1/P of step 2), ncclAllGather
+ *     rebuilds the full f on every rank. Same NVLink bytes, 1/P of the update work.
+ * 0 (default) = ISD when world > 1, else ALLREDUCE. EINVAL for other values. */
+#define LMOSEM_COMBINE_ALLREDUCE 1
+#define LMOSEM_COMBINE_ISD 2
+lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode);
+
+/* The combine mode in effect (-1 for a NULL context). */
+int32_t lmosem_get_combine(const lmosem_ctx* ctx);
 
 /* Out-of-L2 strategy: step 1 runs as z-slab passes when the
  * image is too large for L2 — pass A accumulates each event's forward projection over

@@ -34,6 +34,8 @@ struct lmosem_ctx {
     lmk::GridGeom geom{};
     lmk::BrickIt bricks{};
     int64_t nbf = 0;           // floats per padded brick image (8 * bricks)
+    int64_t nb_alloc = 0;      // bricks allocated: nb rounded up to a multiple of world
+    int combine = 0;           // LMOSEM_COMBINE_* (0 = auto)
     float* c = nullptr;        // error image, bricks (kept all-zero between subsets)
     float* fb = nullptr;       // brick copy of the current f
     float* norm = nullptr;     // s in bricks (halo = 0)
@@ -100,6 +102,11 @@ void block_range(int64_t n, int r, int P, int64_t* b, int64_t* e) {
 int grid_for(lmosem_ctx* ctx, int64_t items) {
     const int64_t cap = (int64_t)ctx->num_sms * 16;
     return (int)std::max<int64_t>(1, std::min<int64_t>((items + 255) / 256, cap));
+}
+
+int combine_mode(const lmosem_ctx* ctx) {
+    if (ctx->combine) return ctx->combine;
+    return ctx->world > 1 ? LMOSEM_COMBINE_ISD : LMOSEM_COMBINE_ALLREDUCE;
 }
 
 lmosem_status launch_to_brick(lmosem_ctx* ctx, const float* row, float* br) {
@@ -183,9 +190,11 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
 }
 
 // step 2 on the bricks; f_row (caller layout) is written when non-null
-lmosem_status launch_update(lmosem_ctx* ctx, float* f_row) {
-    lmk::k_update<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->fb, ctx->c, ctx->norm, f_row, ctx->geom,
-                                                                          ctx->bricks);
+lmosem_status launch_update(lmosem_ctx* ctx, float* f_row, int64_t b_begin = 0, int64_t b_end = -1) {
+    if (b_end < 0) b_end = ctx->bricks.nb;
+    if (b_end <= b_begin) return LMOSEM_OK;
+    lmk::k_update<<<grid_for(ctx, b_end - b_begin), 256, 0, ctx->stream>>>(ctx->fb, ctx->c, ctx->norm, f_row, ctx->geom,
+                                                                           ctx->bricks, b_begin, b_end);
     CK(cudaGetLastError());
     ctx->st.launches++;
     return LMOSEM_OK;
@@ -225,9 +234,25 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
     if ((s = mark(ctx, pm, 1))) return s;
     if ((s = launch_project(ctx, ev + b, e - b, nullptr, 0))) return s;
     if ((s = mark(ctx, pm, 2))) return s;
-    if (ctx->comm) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
-    if ((s = mark(ctx, pm, 3))) return s;
-    if ((s = launch_update(ctx, write_f ? f : nullptr))) return s;
+    if (ctx->comm && combine_mode(ctx) == LMOSEM_COMBINE_ISD) {
+        // PAPER.md lines 509-518 (Listing 3 l.15-19): PSD -> ISD. Reduce-scatter c so rank r
+        // holds the sum over its brick block, update only that block, all-gather f.
+        const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
+        float* my_c = ctx->c + 8 * b0;
+        NK(ncclReduceScatter(ctx->c, my_c, (size_t)(8 * chunk), ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+        if ((s = mark(ctx, pm, 3))) return s;
+        if ((s = launch_update(ctx, nullptr, b0, std::min(b0 + chunk, ctx->bricks.nb)))) return s;  // zeroes own c
+        if (b0 > 0) CK(cudaMemsetAsync(ctx->c, 0, sizeof(float) * 8 * b0, ctx->stream));
+        const int64_t rest = ctx->nb_alloc - (b0 + chunk);
+        if (rest > 0) CK(cudaMemsetAsync(my_c + 8 * chunk, 0, sizeof(float) * 8 * rest, ctx->stream));
+        NK(ncclAllGather(ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk), ncclFloat32, ctx->comm, ctx->stream));
+        if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
+    } else {
+        if (ctx->comm)
+            NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+        if ((s = mark(ctx, pm, 3))) return s;
+        if ((s = launch_update(ctx, write_f ? f : nullptr))) return s;
+    }
     if ((s = mark(ctx, pm, 4))) return s;
     ctx->st.subsets++;
     ctx->st.events += e - b;
@@ -269,7 +294,7 @@ lmosem_status resolve_timing(lmosem_ctx* ctx) {
 
 }  // namespace
 
-LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.3 sm_100a"; }
+LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.4 sm_100a"; }
 
 LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end) {
     if (!begin || !end || n < 0 || world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
@@ -332,6 +357,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     ctx->bricks.BZ = ctx->geom.P[2] / 2;
     ctx->bricks.nb = (int64_t)ctx->bricks.BX * ctx->bricks.BY * ctx->bricks.BZ;
     ctx->nbf = 8 * ctx->bricks.nb;
+    ctx->nb_alloc = (ctx->bricks.nb + world - 1) / world * world;  // equal ISD brick blocks
     if (ctx->nbf >= (int64_t(1) << 31)) {
         delete ctx;
         return LMOSEM_EINVAL;
@@ -384,9 +410,9 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     ctx->stream = ctx->own_stream;
-    cuda(cudaMalloc(&ctx->c, sizeof(float) * ctx->nbf), "cudaMalloc(c)");
-    cuda(cudaMalloc(&ctx->fb, sizeof(float) * ctx->nbf), "cudaMalloc(fb)");
-    cuda(cudaMalloc(&ctx->norm, sizeof(float) * ctx->nbf), "cudaMalloc(norm)");
+    cuda(cudaMalloc(&ctx->c, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(c)");
+    cuda(cudaMalloc(&ctx->fb, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(fb)");
+    cuda(cudaMalloc(&ctx->norm, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(norm)");
     cuda(cudaMalloc(&ctx->scratch, sizeof(float) * V), "cudaMalloc(scratch)");
     for (int k = 0; k < 2; ++k) {
         cuda(cudaEventCreateWithFlags(&ctx->ev_copied[k], cudaEventDisableTiming), "cudaEventCreate");
@@ -394,8 +420,9 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
     if (s != LMOSEM_OK) return bail(s);
     cuda(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * V, cudaMemcpyDefault, ctx->stream), "copy norm");
-    cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * ctx->nbf, ctx->stream), "memset c");
-    cuda(cudaMemsetAsync(ctx->fb, 0, sizeof(float) * ctx->nbf, ctx->stream), "memset fb");
+    cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset c");
+    cuda(cudaMemsetAsync(ctx->fb, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset fb");
+    cuda(cudaMemsetAsync(ctx->norm, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset norm");
     if (s == LMOSEM_OK) {
         lmk::k_row_to_brick<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->scratch, ctx->norm,
                                                                                      ctx->geom, ctx->bricks);
@@ -416,6 +443,15 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     *out = ctx;
     return LMOSEM_OK;
 }
+
+LMOSEM_API lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode) {
+    USABLE(ctx);
+    if (mode < 0 || mode > LMOSEM_COMBINE_ISD) return fail(ctx, LMOSEM_EINVAL, "set_combine: bad mode");
+    ctx->combine = mode;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API int32_t lmosem_get_combine(const lmosem_ctx* ctx) { return ctx ? combine_mode(ctx) : -1; }
 
 LMOSEM_API lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs) {
     USABLE(ctx);

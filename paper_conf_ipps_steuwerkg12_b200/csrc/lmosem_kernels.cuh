@@ -486,10 +486,12 @@ __device__ __forceinline__ float upd1(float f, float c, float s) {
     return (c > 0.0f && s > 0.0f) ? f * __fdiv_rn(c, s) : f;
 }
 
+// Bricks [b_begin, b_end) (the whole image, or this rank's block in the ISD combine).
 __global__ void __launch_bounds__(256) k_update(float* __restrict__ fb, float* __restrict__ cb,
                                                 const float* __restrict__ sb, float* __restrict__ f_row, GridGeom g,
-                                                BrickIt it) {
-    for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
+                                                BrickIt it, int64_t b_begin, int64_t b_end) {
+    for (int64_t b = b_begin + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < b_end;
+         b += (int64_t)gridDim.x * blockDim.x) {
         float4* F = reinterpret_cast<float4*>(fb + 8 * b);
         float4* C = reinterpret_cast<float4*>(cb + 8 * b);
         const float4* S = reinterpret_cast<const float4*>(sb + 8 * b);

@@ -26,8 +26,9 @@ EXPORTS = (
     "lmosem_subset_step", "lmosem_reconstruct", "lmosem_reconstruct_host", "lmosem_error_image",
     "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
     "lmosem_destroy", "lmosem_last_error", "lmosem_set_slabs", "lmosem_get_slabs",
-    "lmosem_sensitivity", "lmosem_set_norm",
+    "lmosem_sensitivity", "lmosem_set_norm", "lmosem_set_combine", "lmosem_get_combine",
 )
+COMBINE_ALLREDUCE, COMBINE_ISD = 1, 2
 
 
 class LmosemError(RuntimeError):
@@ -74,6 +75,8 @@ def load(build_if_missing: bool = False) -> ctypes.CDLL:
         "lmosem_init": ([ctypes.POINTER(_P), _P, _P, _P, ctypes.POINTER(Dist)], _S),
         "lmosem_set_stream": ([_P, _P], _S),
         "lmosem_set_slabs": ([_P, _I32], _S),
+        "lmosem_set_combine": ([_P, _I32], _S),
+        "lmosem_get_combine": ([_P], _I32),
         "lmosem_get_slabs": ([_P], _I32),
         "lmosem_subset_step": ([_P, _P, _I64, _P], _S),
         "lmosem_reconstruct": ([_P, _P, _P, _I32, _I32, _P], _S),
@@ -265,6 +268,14 @@ class Reconstructor:
 
     def update(self, f, c):
         self._check(self._lib.lmosem_update(self._h, _dev_ptr(f, "float32", self.V), _dev_ptr(c, "float32", self.V)))
+
+    def set_combine(self, mode: int):
+        """0 = auto, COMBINE_ALLREDUCE or COMBINE_ISD (see lmosem.h)."""
+        self._check(self._lib.lmosem_set_combine(self._h, int(mode)))
+
+    @property
+    def combine(self) -> int:
+        return int(self._lib.lmosem_get_combine(self._h))
 
     def set_slabs(self, n_slabs: int):
         """z-slab passes for step 1 (0 = automatic from the L2 budget); see lmosem.h."""

@@ -52,6 +52,17 @@ def _worker(rank, world, port, q):
         same = all(torch.equal(gathered[0], x) for x in gathered)
         f_one = oracle.subset_step(g, ev, s, f0)
         err = float(np.max(np.abs(f_dist - f_one) / f_one))
+        # ISD step 2: rank r updates only its block of the image
+        # from the summed c, then the blocks are all-gathered into the full f
+        V = cfg.n_voxels
+        assert V % world == 0
+        blk = V // world
+        vb = rank * blk
+        f_block = torch.from_numpy(oracle.update(f0[vb:vb + blk], c.numpy()[vb:vb + blk], s[vb:vb + blk]))
+        parts = [torch.empty(blk, dtype=torch.float64) for _ in range(world)]
+        dist.all_gather(parts, f_block)
+        f_isd = torch.cat(parts).numpy()
+        err = max(err, float(np.max(np.abs(f_isd - f_one) / f_one)))
         # NCCL-id broadcast plumbing used by the GPU path
         d = pkg.make_dist(rank, world)
         ids = [None] * world

@@ -407,3 +407,27 @@ def test_nccl_combine_single_rank(pkg):
     torch.testing.assert_close(f1, f0, rtol=1e-6, atol=0)
     rec0.close()
     rec1.close()
+
+
+@pytest.mark.parametrize("combine", [1, 2])
+def test_combine_modes_single_rank(pkg, combine):
+    """Both combines on a 1-rank communicator — all-reduce + full update, and the paper's
+    PSD -> ISD switch (reduce-scatter, block update, all-gather) —
+    through subset_step and a multi-subset reconstruct, against the oracle."""
+    cfg, ev, s = inputs("C1")
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), dist=(0, 1, pkg.nccl_unique_id()))
+    rec.set_combine(combine)
+    assert rec.combine == combine
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.subset_step(dev(ev[:cfg.n_events]), f)
+    rec.synchronize()
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    ref = oracle.subset_step(g, ev[:cfg.n_events], s, np.ones(cfg.n_voxels))
+    assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
+    f2 = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(dev(ev), off, 2, f2)
+    rec.synchronize()
+    ref2 = oracle.reconstruct(g, ev, off, 2, s, np.ones(cfg.n_voxels))
+    assert rel_l2(f2.cpu().numpy().astype(np.float64), ref2) <= REL_L2_RECON
+    rec.close()
