@@ -102,12 +102,12 @@ lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
 
 /* Creates a context on the current CUDA device.
  *   dims[3]     = {nx, ny, nz} > 0, V < 2^31
- *   voxel_mm[3] = voxel size in mm, finite and > 0
+ *   voxel_mm[3] = voxel size in mm, finite and > 0 (float64: the geometry is float64)
  *   norm        = V float32 sensitivity image s (device or host); copied, caller keeps it
  *   dist        = NULL for one GPU, else the rank/world/NCCL id (collective init;
  *                 EINVAL if world < 1, rank outside [0, world) or the id is NULL)
  * Returns EINVAL / ENOMEM / ECUDA / ENCCL; *out is NULL on failure. */
-lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
+lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3],
                           const float* norm, const lmosem_dist* dist);
 
 /* Combine of the per-GPU error images (world > 1; needs a context created with a dist):

@@ -29,7 +29,7 @@ struct PhaseMarks {
 struct lmosem_ctx {
     int device = -1;
     int32_t dims[3] = {0, 0, 0};
-    float vox[3] = {0, 0, 0};
+    double vox[3] = {0, 0, 0};
     int64_t V = 0;
     lmk::GridGeom geom{};
     lmk::BrickIt bricks{};
@@ -310,7 +310,7 @@ LMOSEM_API lmosem_status lmosem_nccl_unique_id(void* out, size_t size) {
     return LMOSEM_OK;
 }
 
-LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const float voxel_mm[3],
+LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3],
                                      const float* norm, const lmosem_dist* dist) {
     if (!out) return LMOSEM_EINVAL;
     *out = nullptr;
@@ -318,7 +318,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     int64_t V = 1;
     for (int k = 0; k < 3; ++k) {
         if (dims[k] <= 0) return LMOSEM_EINVAL;
-        if (!std::isfinite(voxel_mm[k]) || !(voxel_mm[k] > 0.0f)) return LMOSEM_EINVAL;
+        if (!std::isfinite(voxel_mm[k]) || !(voxel_mm[k] > 0.0)) return LMOSEM_EINVAL;
         V *= dims[k];
     }
     if (V >= (int64_t(1) << 31)) return LMOSEM_EINVAL;
@@ -343,8 +343,8 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         ctx->dims[k] = dims[k];
         ctx->vox[k] = voxel_mm[k];
         ctx->geom.n[k] = dims[k];
-        ctx->geom.lo[k] = -0.5 * (double)dims[k] * (double)voxel_mm[k];
-        ctx->geom.inv_v[k] = 1.0 / (double)voxel_mm[k];
+        ctx->geom.lo[k] = -0.5 * (double)dims[k] * voxel_mm[k];
+        ctx->geom.inv_v[k] = 1.0 / voxel_mm[k];
     }
     for (int k = 0; k < 3; ++k) {
         ctx->geom.clo[k] = 0;

@@ -167,7 +167,7 @@ class Reconstructor:
         self.voxel_mm = tuple(float(v) for v in voxel_mm)
         self.V = self.dims[0] * self.dims[1] * self.dims[2]
         d = (ctypes.c_int32 * 3)(*self.dims)
-        v = (ctypes.c_float * 3)(*self.voxel_mm)
+        v = (ctypes.c_double * 3)(*self.voxel_mm)
         if isinstance(norm, torch.Tensor) and norm.is_cuda:
             nptr = _dev_ptr(norm, "float32", self.V)
             torch.cuda.current_stream().synchronize()

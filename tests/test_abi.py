@@ -63,7 +63,7 @@ def test_block_range_einval(lib, args):
 def _init(lib, dims, vox, norm_ptr=1, dist=None):
     h = ctypes.c_void_p(123)
     d = (ctypes.c_int32 * 3)(*dims)
-    v = (ctypes.c_float * 3)(*vox)
+    v = (ctypes.c_double * 3)(*vox)
     st = lib.lmosem_init(ctypes.byref(h), d, v, norm_ptr, dist)
     return st, h
 
@@ -79,7 +79,7 @@ def test_init_einval_before_cuda(lib, dims, vox):
 def test_init_einval_pointers_and_dist(lib):
     h = ctypes.c_void_p()
     d = (ctypes.c_int32 * 3)(4, 4, 4)
-    v = (ctypes.c_float * 3)(1, 1, 1)
+    v = (ctypes.c_double * 3)(1, 1, 1)
     assert lib.lmosem_init(None, d, v, 1, None) == L.EINVAL
     assert lib.lmosem_init(ctypes.byref(h), None, v, 1, None) == L.EINVAL
     assert lib.lmosem_init(ctypes.byref(h), d, v, None, None) == L.EINVAL
