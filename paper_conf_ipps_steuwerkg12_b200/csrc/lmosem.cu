@@ -43,6 +43,8 @@ struct lmosem_ctx {
     int cap = 0;               // path-piece capacity per warp
     int slabs_forced = 0;      // z-slab count (0 = automatic from the L2 budget)
     float* fp_acc = nullptr;   // per-event forward projections of the z-slab passes
+    unsigned long long* work = nullptr;  // k_project work counters (one per launch in a step)
+    int work_next = 0;
     int64_t fp_cap = 0;
     size_t proj_smem = 0;      // dynamic shared memory of k_project
     cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
@@ -134,19 +136,27 @@ int n_slabs(const lmosem_ctx* ctx) {
     return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
 }
 
+constexpr int kWorkSlots = 1024;  // counters, reused round-robin (zeroed per launch)
+
 lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
-    const int64_t warps_needed = (n + 31) / 32;
     const int64_t wpb = lmk::PROJ_THREADS / 32;
-    const int64_t blocks_needed = (warps_needed + wpb - 1) / wpb;
+    const int64_t resident = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm * wpb;
+    // events per claim: 32 when every warp gets >= 4 claims, else smaller (>= 4)
+    int batch = 32;
+    while (batch > 4 && n < (int64_t)batch * resident * 4) batch >>= 1;
+    const int64_t blocks_needed = ((n + batch - 1) / batch + wpb - 1) / wpb;
     const int64_t cap = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm;
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
     const size_t sm = ctx->proj_smem;
+    unsigned long long* work = ctx->work + ctx->work_next;
+    ctx->work_next = (ctx->work_next + 1) % kWorkSlots;
+    CK(cudaMemsetAsync(work, 0, sizeof(unsigned long long), ctx->stream));
     switch (mode) {
-        case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
-        case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
-        case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
-        case 3: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
-        default: lmk::k_project<4><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap); break;
+        case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
+        case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
+        case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
+        case 3: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
+        default: lmk::k_project<4><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
     }
     CK(cudaGetLastError());
     ctx->st.launches++;
@@ -414,6 +424,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cuda(cudaMalloc(&ctx->fb, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(fb)");
     cuda(cudaMalloc(&ctx->norm, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(norm)");
     cuda(cudaMalloc(&ctx->scratch, sizeof(float) * V), "cudaMalloc(scratch)");
+    cuda(cudaMalloc(&ctx->work, sizeof(unsigned long long) * kWorkSlots), "cudaMalloc(work)");
     for (int k = 0; k < 2; ++k) {
         cuda(cudaEventCreateWithFlags(&ctx->ev_copied[k], cudaEventDisableTiming), "cudaEventCreate");
         cuda(cudaEventCreateWithFlags(&ctx->ev_consumed[k], cudaEventDisableTiming), "cudaEventCreate");
@@ -664,6 +675,7 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (ctx->norm) cudaFree(ctx->norm);
     if (ctx->scratch) cudaFree(ctx->scratch);
     if (ctx->fp_acc) cudaFree(ctx->fp_acc);
+    if (ctx->work) cudaFree(ctx->work);
     if (ctx->own_stream) cudaStreamDestroy(ctx->own_stream);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     delete ctx;

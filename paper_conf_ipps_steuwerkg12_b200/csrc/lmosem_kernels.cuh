@@ -337,7 +337,8 @@ constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 template <int MODE>
 __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
-                                                             float* __restrict__ fp, GridGeom g, int cap) {
+                                                             float* __restrict__ fp, GridGeom g, int cap,
+                                                             unsigned long long* __restrict__ work, int batch) {
     constexpr bool kGather = MODE <= 2;    // forward projection in this launch
     constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4;  // back-projection in this launch
     constexpr bool kStore = kScatter && !LMK_RECOMPUTE;  // keep pieces for the scatter pass
@@ -346,14 +347,20 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
     const int wib = threadIdx.x >> 5;
     const unsigned path_s = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)wib * cap);
     const unsigned lt = (1u << lane) - 1u;
-    const int64_t warp = (int64_t)blockIdx.x * (blockDim.x >> 5) + wib;
-    const int64_t nwarps = (int64_t)gridDim.x * (blockDim.x >> 5);
-    for (int64_t base = warp * 32; base < n; base += nwarps * 32) {
+    // dynamic work distribution: each warp claims `batch` (<= 32) consecutive events at a
+    // time from a global counter (zeroed before the launch), so unequal LOR lengths and
+    // small per-rank subsets do not leave a tail of idle warps
+    for (;;) {
+        unsigned long long claim = 0;
+        if (lane == 0) claim = atomicAdd(work, (unsigned long long)batch);
+        const int64_t base = (int64_t)__shfl_sync(0xffffffffu, claim, 0);
+        if (base >= n) break;
         const int64_t idx = base + lane;
+        const bool mine_ev = lane < batch && idx < n;
         Lor mine;
         bool ok = false;
         float fp_known = 1.0f;  // MODE 4 back-projects len * 1
-        if (idx < n) {
+        if (mine_ev) {
             float ev[6];
             load_event(events, idx, ev);
             ok = lor_setup(ev, g, mine);
@@ -362,7 +369,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 ok = ok && fp_known > 0.0f;  // reading S7
             }
         }
-        if (MODE == 1 && idx < n && !ok) fp[idx] = 0.0f;
+        if (MODE == 1 && mine_ev && !ok) fp[idx] = 0.0f;
         unsigned mask = __ballot_sync(0xffffffffu, ok);
         while (mask) {
             const int src = __ffs(mask) - 1;
