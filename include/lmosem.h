@@ -174,8 +174,9 @@ lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* events, int64_
  * gets the full image). Stream-ordered. */
 lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events, float* s_out);
 
-/* Replaces the context's norm image s (V float32, device or host; copied). Stream-ordered:
- * later calls use the new s. EINVAL for NULL. */
+/* Replaces the context's norm image s (V float32, device or host; copied). Waits for the
+ * copy, so the caller may release `norm` on return; later calls use the new s. EINVAL for
+ * NULL. */
 lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm);
 
 /* Step 2 only, for tests: f_j <- f_j*c_j/s_j where c_j > 0 and s_j > 0 (device f and c,

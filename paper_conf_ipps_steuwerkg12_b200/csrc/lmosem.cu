@@ -50,7 +50,7 @@ struct lmosem_ctx {
     cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
     int rank = 0, world = 1;
     ncclComm_t comm = nullptr;
-    int num_sms = 0, proj_blocks_per_sm = 0, upd_blocks = 0;
+    int num_sms = 0, proj_blocks_per_sm = 0;
     bool failed = false;
     std::string err;
     // timing
@@ -416,7 +416,6 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
                                                        ctx->proj_smem),
          "occupancy");
     if (ctx->proj_blocks_per_sm < 1) ctx->proj_blocks_per_sm = 1;
-    ctx->upd_blocks = ctx->num_sms * 8;
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     ctx->stream = ctx->own_stream;
@@ -605,7 +604,10 @@ LMOSEM_API lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm) {
     USABLE(ctx);
     if (!norm) return fail(ctx, LMOSEM_EINVAL, "set_norm: null norm");
     CK(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * ctx->V, cudaMemcpyDefault, ctx->stream));
-    return launch_to_brick(ctx, ctx->scratch, ctx->norm);
+    lmosem_status s = launch_to_brick(ctx, ctx->scratch, ctx->norm);
+    if (s) return s;
+    CK(cudaStreamSynchronize(ctx->stream));  // the caller may release `norm` on return
+    return LMOSEM_OK;
 }
 
 LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {

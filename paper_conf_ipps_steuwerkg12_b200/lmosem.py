@@ -263,8 +263,6 @@ class Reconstructor:
         else:
             ptr = _host_ptr(norm, self.V)
         self._check(self._lib.lmosem_set_norm(self._h, ptr))
-        if not (isinstance(norm, torch.Tensor) and norm.is_cuda):
-            self.synchronize()  # the host buffer may be released by the caller
 
     def update(self, f, c):
         self._check(self._lib.lmosem_update(self._h, _dev_ptr(f, "float32", self.V), _dev_ptr(c, "float32", self.V)))
