@@ -61,7 +61,8 @@ typedef enum {
     LMOSEM_ENOMEM = 2,
     LMOSEM_ECUDA = 3,
     LMOSEM_ENCCL = 4,
-    LMOSEM_ESTATE = 5
+    LMOSEM_ESTATE = 5,
+    LMOSEM_EIO = 6
 } lmosem_status;
 
 #define LMOSEM_NCCL_ID_BYTES 128
@@ -156,6 +157,17 @@ lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event* events, co
  * double-buffered so the upload of subset l+1 overlaps the projection of subset l,
  * downloads f. Synchronous. */
 lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
+                                      int32_t n_subsets, int32_t n_iterations, float* f);
+
+/* As lmosem_reconstruct with the events read from a list-mode file (Listing 2
+ * lines 2-3, read_events per subset): `path` is a raw array of lmosem_event records
+ * (24 B each, native-endian float32, no header); subset l is records
+ * [offsets[l], offsets[l+1]). Each rank reads only its block of every subset with pread
+ * into double-buffered pinned staging buffers (context-owned), so the file read and the
+ * H2D copy of subset l+1 overlap the projection of subset l. f: V float32 DEVICE image
+ * (in: f0, out: result). Synchronous. EIO if the file cannot be opened or read or is
+ * shorter than offsets[n_subsets] records (the context stays usable after EIO). */
+lmosem_status lmosem_reconstruct_file(lmosem_ctx* ctx, const char* path, const int64_t* offsets,
                                       int32_t n_subsets, int32_t n_iterations, float* f);
 
 /* Step 1 only, for tests: c_out (V float32, device) <- error image of n_events device

@@ -3,7 +3,12 @@
 #include <cuda_runtime.h>
 #include <nccl.h>
 
+#include <fcntl.h>
+#include <sys/stat.h>
+#include <unistd.h>
+
 #include <algorithm>
+#include <cerrno>
 #include <cmath>
 #include <cstdio>
 #include <cstring>
@@ -63,6 +68,9 @@ struct lmosem_ctx {
     int64_t dev_ev_cap = 0;
     float* dev_f = nullptr;
     cudaEvent_t ev_copied[2] = {nullptr, nullptr}, ev_consumed[2] = {nullptr, nullptr};
+    // file streaming: pinned staging buffers
+    lmosem_event* pin_ev[2] = {nullptr, nullptr};
+    int64_t pin_cap = 0;
 };
 
 namespace {
@@ -500,12 +508,10 @@ LMOSEM_API lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event*
     return LMOSEM_OK;
 }
 
-LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
-                                                 int32_t n_subsets, int32_t n_iterations, float* f) {
-    USABLE(ctx);
-    if (!f || n_iterations < 0 || check_offsets(offsets, n_subsets) || (offsets[n_subsets] > offsets[0] && !events))
-        return fail(ctx, LMOSEM_EINVAL, "reconstruct_host: bad arguments");
-    // this rank's block of every subset: the only events it uploads (block distribution)
+namespace {
+
+// Device double buffers for streamed subsets (this rank's largest block).
+lmosem_status ensure_stream_buffers(lmosem_ctx* ctx, const int64_t* offsets, int32_t n_subsets, bool pinned) {
     int64_t cap = 1;
     for (int32_t l = 0; l < n_subsets; ++l) {
         int64_t b, e;
@@ -521,6 +527,104 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
         for (int k = 0; k < 2; ++k) CK(cudaMalloc(&ctx->dev_ev[k], sizeof(lmosem_event) * cap));
         ctx->dev_ev_cap = cap;
     }
+    if (pinned && cap > ctx->pin_cap) {
+        for (int k = 0; k < 2; ++k) {
+            if (ctx->pin_ev[k]) CK(cudaFreeHost(ctx->pin_ev[k]));
+            ctx->pin_ev[k] = nullptr;
+        }
+        ctx->pin_cap = 0;
+        for (int k = 0; k < 2; ++k) CK(cudaHostAlloc(&ctx->pin_ev[k], sizeof(lmosem_event) * cap, cudaHostAllocDefault));
+        ctx->pin_cap = cap;
+    }
+    return LMOSEM_OK;
+}
+
+// Reads exactly `bytes` at `off` (retries short reads and EINTR).
+bool pread_all(int fd, void* dst, size_t bytes, off_t off) {
+    char* p = static_cast<char*>(dst);
+    while (bytes > 0) {
+        const ssize_t r = pread(fd, p, bytes, off);
+        if (r < 0 && errno == EINTR) continue;
+        if (r <= 0) return false;
+        p += r;
+        off += r;
+        bytes -= (size_t)r;
+    }
+    return true;
+}
+
+}  // namespace
+
+LMOSEM_API lmosem_status lmosem_reconstruct_file(lmosem_ctx* ctx, const char* path, const int64_t* offsets,
+                                                 int32_t n_subsets, int32_t n_iterations, float* f) {
+    USABLE(ctx);
+    if (!path || !f || n_iterations < 0 || check_offsets(offsets, n_subsets))
+        return fail(ctx, LMOSEM_EINVAL, "reconstruct_file: bad arguments");
+    const int fd = open(path, O_RDONLY);
+    if (fd < 0) return fail(ctx, LMOSEM_EIO, std::string("reconstruct_file: open ") + path + ": " + strerror(errno));
+    struct stat sb;
+    if (fstat(fd, &sb) != 0 || (int64_t)sb.st_size < offsets[n_subsets] * (int64_t)sizeof(lmosem_event)) {
+        close(fd);
+        return fail(ctx, LMOSEM_EIO, std::string("reconstruct_file: ") + path + " is shorter than offsets[n_subsets]");
+    }
+    lmosem_status s = ensure_stream_buffers(ctx, offsets, n_subsets, true);
+    if (s) {
+        close(fd);
+        return s;
+    }
+    // staging buffer k is free once the H2D copy out of it (ev_copied[k]) completed;
+    // device buffer k is free once the projection of its subset (ev_consumed[k]) completed
+    for (int k = 0; k < 2; ++k) {
+        if (cudaEventRecord(ctx->ev_consumed[k], ctx->stream) != cudaSuccess ||
+            cudaEventRecord(ctx->ev_copied[k], ctx->copy_stream) != cudaSuccess) {
+            close(fd);
+            return fail(ctx, LMOSEM_ECUDA, "reconstruct_file: cudaEventRecord");
+        }
+    }
+    int64_t step = 0;
+    const int64_t total = (int64_t)n_iterations * n_subsets;
+    for (int32_t it = 0; it < n_iterations && !s; ++it)
+        for (int32_t l = 0; l < n_subsets && !s; ++l, ++step) {
+            const int k = (int)(step & 1);
+            int64_t b, e;
+            block_range(offsets[l + 1] - offsets[l], ctx->rank, ctx->world, &b, &e);
+            // host: read this rank's block while the GPU works on the previous subset
+            if (cudaEventSynchronize(ctx->ev_copied[k]) != cudaSuccess) {
+                s = fail(ctx, LMOSEM_ECUDA, "reconstruct_file: staging sync");
+                break;
+            }
+            if (e > b && !pread_all(fd, ctx->pin_ev[k], sizeof(lmosem_event) * (e - b),
+                                    (off_t)(sizeof(lmosem_event) * (offsets[l] + b)))) {
+                s = fail(ctx, LMOSEM_EIO, std::string("reconstruct_file: read ") + path + ": " + strerror(errno));
+                break;
+            }
+            if (cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_consumed[k], 0) != cudaSuccess ||
+                (e > b && cudaMemcpyAsync(ctx->dev_ev[k], ctx->pin_ev[k], sizeof(lmosem_event) * (e - b),
+                                          cudaMemcpyHostToDevice, ctx->copy_stream) != cudaSuccess) ||
+                cudaEventRecord(ctx->ev_copied[k], ctx->copy_stream) != cudaSuccess ||
+                cudaStreamWaitEvent(ctx->stream, ctx->ev_copied[k], 0) != cudaSuccess) {
+                s = fail(ctx, LMOSEM_ECUDA, "reconstruct_file: upload");
+                break;
+            }
+            s = subset_iteration(ctx, ctx->dev_ev[k], e - b, f, false, step == 0, step == total - 1);
+            if (!s && cudaEventRecord(ctx->ev_consumed[k], ctx->stream) != cudaSuccess)
+                s = fail(ctx, LMOSEM_ECUDA, "reconstruct_file: cudaEventRecord");
+        }
+    close(fd);
+    if (s == LMOSEM_EIO) cudaStreamSynchronize(ctx->stream);  // nothing left in flight on return
+    if (s) return s;
+    CK(cudaStreamSynchronize(ctx->stream));
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
+                                                 int32_t n_subsets, int32_t n_iterations, float* f) {
+    USABLE(ctx);
+    if (!f || n_iterations < 0 || check_offsets(offsets, n_subsets) || (offsets[n_subsets] > offsets[0] && !events))
+        return fail(ctx, LMOSEM_EINVAL, "reconstruct_host: bad arguments");
+    // this rank's block of every subset: the only events it uploads (block distribution)
+    lmosem_status s0 = ensure_stream_buffers(ctx, offsets, n_subsets, false);
+    if (s0) return s0;
     if (!ctx->dev_f) CK(cudaMalloc(&ctx->dev_f, sizeof(float) * ctx->V));
     CK(cudaMemcpyAsync(ctx->dev_f, f, sizeof(float) * ctx->V, cudaMemcpyHostToDevice, ctx->stream));
     // buffers start free
@@ -667,6 +771,7 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     for (auto e : ctx->h2d_pending) cudaEventDestroy(e);
     for (auto e : ctx->h2d_pool) cudaEventDestroy(e);
     for (int k = 0; k < 2; ++k) {
+        if (ctx->pin_ev[k]) cudaFreeHost(ctx->pin_ev[k]);
         if (ctx->dev_ev[k]) cudaFree(ctx->dev_ev[k]);
         if (ctx->ev_copied[k]) cudaEventDestroy(ctx->ev_copied[k]);
         if (ctx->ev_consumed[k]) cudaEventDestroy(ctx->ev_consumed[k]);

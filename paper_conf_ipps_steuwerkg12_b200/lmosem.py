@@ -16,8 +16,8 @@ _PKG = os.path.dirname(os.path.abspath(__file__))
 # LMOSEM_LIB selects an in-tree A/B build of the same library (tools/ab_variants.py)
 SO_PATH = os.environ.get("LMOSEM_LIB") or os.path.join(_PKG, "liblmosem.so")
 
-OK, EINVAL, ENOMEM, ECUDA, ENCCL, ESTATE = range(6)
-_NAMES = {0: "OK", 1: "EINVAL", 2: "ENOMEM", 3: "ECUDA", 4: "ENCCL", 5: "ESTATE"}
+OK, EINVAL, ENOMEM, ECUDA, ENCCL, ESTATE, EIO = range(7)
+_NAMES = {0: "OK", 1: "EINVAL", 2: "ENOMEM", 3: "ECUDA", 4: "ENCCL", 5: "ESTATE", 6: "EIO"}
 NCCL_ID_BYTES = 128
 
 # every symbol include/lmosem.h declares (checked by tests/test_abi.py)
@@ -27,6 +27,7 @@ EXPORTS = (
     "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
     "lmosem_destroy", "lmosem_last_error", "lmosem_set_slabs", "lmosem_get_slabs",
     "lmosem_sensitivity", "lmosem_set_norm", "lmosem_set_combine", "lmosem_get_combine",
+    "lmosem_reconstruct_file",
 )
 COMBINE_ALLREDUCE, COMBINE_ISD = 1, 2
 
@@ -81,6 +82,7 @@ def load(build_if_missing: bool = False) -> ctypes.CDLL:
         "lmosem_subset_step": ([_P, _P, _I64, _P], _S),
         "lmosem_reconstruct": ([_P, _P, _P, _I32, _I32, _P], _S),
         "lmosem_reconstruct_host": ([_P, _P, _P, _I32, _I32, _P], _S),
+        "lmosem_reconstruct_file": ([_P, ctypes.c_char_p, _P, _I32, _I32, _P], _S),
         "lmosem_error_image": ([_P, _P, _I64, _P, _P], _S),
         "lmosem_forward": ([_P, _P, _I64, _P, _P], _S),
         "lmosem_update": ([_P, _P, _P], _S),
@@ -239,6 +241,12 @@ class Reconstructor:
         off = np.ascontiguousarray(offsets, dtype=np.int64)
         self._check(self._lib.lmosem_reconstruct_host(self._h, _host_ptr(events), off.ctypes.data, off.size - 1,
                                                       int(n_iterations), _host_ptr(f, self.V)))
+
+    def reconstruct_file(self, path, offsets, n_iterations, f):
+        """Events streamed from a raw lmosem_event file (24 B records), f a CUDA tensor."""
+        off = np.ascontiguousarray(offsets, dtype=np.int64)
+        self._check(self._lib.lmosem_reconstruct_file(self._h, os.fsencode(path), off.ctypes.data, off.size - 1,
+                                                      int(n_iterations), _dev_ptr(f, "float32", self.V)))
 
     def error_image(self, events, f, c_out):
         ep, n = self._events_ptr(events)

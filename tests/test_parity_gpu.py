@@ -466,3 +466,32 @@ def test_odd_extents_anisotropic_voxels(pkg, dims, vox):
     ref = oracle.subset_step(g, ev, s, f0.astype(np.float32))
     assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
     rec.close()
+
+
+# ------------------------------------------------------------------ list-mode file streaming (NEXT-4)
+def test_reconstruct_file_matches_device(pkg, tmp_path):
+    """PAPER.md Listing 2 l.2-3 (read_events per subset): events streamed from a raw
+    list-mode file (pread into pinned double buffers) give the device-resident result."""
+    cfg, ev, s = inputs("C1")
+    path = tmp_path / "c1.lm"
+    ev.tofile(path)
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    fd = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(dev(ev), off, 2, fd)
+    ff = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct_file(str(path), off, 2, ff)
+    rec.synchronize()
+    torch.testing.assert_close(ff, fd, rtol=1e-5, atol=0)
+    # errors: missing file, file shorter than the offsets -> EIO, context still usable
+    with pytest.raises(pkg.LmosemError) as e:
+        rec.reconstruct_file(str(tmp_path / "missing.lm"), off, 1, ff)
+    assert e.value.status == 6
+    short = tmp_path / "short.lm"
+    ev[:cfg.n_events].tofile(short)
+    with pytest.raises(pkg.LmosemError) as e:
+        rec.reconstruct_file(str(short), off, 1, ff)
+    assert e.value.status == 6
+    rec.subset_step(dev(ev[:cfg.n_events]), ff)
+    rec.synchronize()
+    rec.close()

@@ -10,7 +10,8 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 VARIANTS = {
     "default": [],
-    "nopipe": ["LMK_PIPE_GATHER=0"],
+    "c256x4": ["LMK_MIN_BLOCKS=4"],
+    "c192x5": ["LMK_CTA_THREADS=192", "LMK_MIN_BLOCKS=5"],
 }
 
 
