@@ -324,12 +324,13 @@ def main():
     proj_avg_s = proj_ms / K * 1e-3
     l2 = l2_peak_gbs(cfg.n_voxels)
     alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0  # 4 B gather + 4 B RED per path element, 24 B/event
-    traffic = None
+    traffic, sectors = None, None
     try:
         with open(os.path.join(ROOT, "profiles", "r01_traffic.json")) as fh:
             t = json.load(fh).get(name)
         if t:
             traffic = t["dram_bytes_read_per_launch"] + t["dram_bytes_write_per_launch"]
+            sectors = t["l2_sectors_read_per_launch"] + t["l2_sectors_red_per_launch"]
     except (OSError, ValueError, KeyError):
         pass
     roof = {"kernel": "k_project<0> (fused Siddon + forward + back-projection)", "bound": "l2",
@@ -346,6 +347,18 @@ def main():
         roof["frac"] = roof["achieved"] / roof["peak"]
         roof["frac_vs_random_pairs"] = roof["achieved"] / (l2["pair"] * 8.0 / 1e9)
         roof["l2_micro_ops_per_s"] = l2
+    roof_sec = None
+    if l2 and sectors:
+        # sector view: the L2 moves 32-byte sectors; both microbenchmarks (random and fully
+        # coalesced gather+RED pairs) saturate at the same sector rate
+        peak_sec = max(l2["red"], l2["ldg"], l2["pair"] * 2.0, l2["pair_run8"] * 2.0 / 8.0,
+                       l2["pair_warp32"] * 2.0 / 8.0)
+        roof_sec = {"bound": "l2_sectors", "achieved": sectors / proj_avg_s, "peak": peak_sec, "unit": "sectors/s",
+                    "frac": sectors / proj_avg_s / peak_sec, "sectors_per_launch": sectors,
+                    "path_elements_per_sector": 2 * pairs / sectors,
+                    "what": "ncu L2 sectors of k_project (gathers + REDs, profiles/r01_traffic.json) / live duration, "
+                            "vs the max sector rate over the live L2 microbenchmark modes (random RED, random gather, "
+                            "random / 8-lane / 32-lane gather+RED pairs)"}
     hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0) / proj_avg_s / 1e9, "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
     hbm["frac"] = hbm["achieved"] / hbm["peak"]
@@ -369,7 +382,7 @@ def main():
                         "CUDA events around each call on the library's stream",
         "phase_ms_per_step": {"convert_f": conv_ms / K, "project": proj_ms / K, "combine": comb_ms / K,
                               "update": upd_ms / K},
-        "roofline": roof, "roofline_hbm_events": hbm, "roofline_update": upd,
+        "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_hbm_events": hbm, "roofline_update": upd,
         "gpu_launches": launches, "flushed_subset_step": flushed,
         "clocks": clk.summary(), "wall_s_timed_region": t_wall,
         "e2e": e2e,
