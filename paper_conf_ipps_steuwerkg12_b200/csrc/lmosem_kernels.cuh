@@ -2,17 +2,17 @@
 //
 // Step 1 (Listing 2 lines 5-13) is ONE fused kernel per subset, k_project: a
 // warp owns one line of response (LOR) at a time:
-//   - setup, per LOR in float64 (one lane per event of a 32-event batch, broadcast by
-//     shuffles): clip to the volume, dominant axis a (largest |du_a| in voxel units),
-//     minor-axis positions at the first slab plane and slopes du_b/du_a, du_c/du_a
-//     (|slope| <= 1), the positions kept in Q24.40 fixed point;
-//   - pass 1 (geometry): lane k takes slabs k, k+32, ... of the dominant axis. Each minor
-//     axis crosses at most one plane inside a slab, so a slab holds <= 3 pieces; the
-//     minor positions at the slab plane are one 64-bit integer multiply-add and the
-//     crossings are float32 relative to that plane (values in [0,1], ~1e-7 voxel absolute
-//     error wherever the slab lies). The pieces (j, len) are compacted into the warp's
-//     shared-memory path buffer in path order; f is gathered for them in the same loop
-//     (the loads of one slab batch complete while the next batch is computed);
+//   - work: warps claim batches of <= 32 events from a global counter; one lane per event
+//     does the float64 setup — clip to the volume, dominant axis a (largest |du_a| in
+//     voxel units), minor-axis positions at the first slab plane and slopes du_b/du_a,
+//     du_c/du_a (|slope| <= 1) in Q24.40 fixed point — broadcast to the warp by shuffles;
+//   - pass 1 (geometry): lane k takes slabs k, k+32, ... of the dominant axis, stepping
+//     its minor positions by exactly 32 slopes (integer adds). Each minor axis crosses at
+//     most one plane inside a slab, so a slab holds <= 3 pieces; up-moving axes are kept
+//     mirrored so the distance to the next plane is the 40-bit fraction, converted to
+//     float exactly (crossings in [0,1] carry ~1e-7 voxel absolute error wherever the slab
+//     lies). The pieces (j, len) are compacted into the warp's shared-memory path buffer
+//     in path order, and f is gathered for them in the same loop;
 //   - forward projection (lines 9-10): a warp reduction of the gathered f*len gives fp;
 //   - pass 2 (back-projection, lines 12-13): lane m reads piece m and issues
 //     red.global.add.f32 of len/fp into c; lanes hold consecutive pieces of one path, so
@@ -319,9 +319,6 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
-#ifndef LMK_RECOMPUTE
-#define LMK_RECOMPUTE 0      // 1: back-projection recomputes the geometry (no shared path buffer)
-#endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 
 // Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2.
@@ -341,7 +338,6 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                                                              unsigned long long* __restrict__ work, int batch) {
     constexpr bool kGather = MODE <= 2;    // forward projection in this launch
     constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4;  // back-projection in this launch
-    constexpr bool kStore = kScatter && !LMK_RECOMPUTE;  // keep pieces for the scatter pass
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
@@ -387,7 +383,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 const bool in = k < L.ns;  // lanes past the last slab compute garbage, store nothing
                 const Pieces P = slab_pieces(L, W, k, S.wb, S.wc, S.Ja);
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
-                if (kStore) append3(path_s, cnt, lt, P, v0, v1, v2);
+                if (kScatter) append3(path_s, cnt, lt, P, v0, v1, v2);
                 if (kGather) {
                     acc = fmaf(v0 ? __ldg(fb + P.j0) : 0.f, P.l0, acc);
                     acc = fmaf(v1 ? __ldg(fb + P.j1) : 0.f, P.l1, acc);
@@ -407,21 +403,10 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
                 // pass 2: back-projection, lane m <- piece m (path order: consecutive
                 // lanes share 32-byte brick sectors)
                 const float inv = 1.0f / fpv;
-                if (kStore) {
 #pragma unroll 8
-                    for (int m = lane; m < cnt; m += 32) {
-                        const int2 q = lds2(path_s + 8u * (unsigned)m);
-                        atomicAdd(cb + q.x, __int_as_float(q.y) * inv);
-                    }
-                } else {
-                    Step S = make_step(L, W, lane);
-                    for (int k0 = 0; k0 < L.ns; k0 += 32, advance(S)) {
-                        const bool in = k0 + lane < L.ns;
-                        const Pieces P = slab_pieces(L, W, k0 + lane, S.wb, S.wc, S.Ja);
-                        if (in && P.l0 > 0.0f) atomicAdd(cb + P.j0, P.l0 * inv);
-                        if (in && P.l1 > 0.0f) atomicAdd(cb + P.j1, P.l1 * inv);
-                        if (in && P.l2 > 0.0f) atomicAdd(cb + P.j2, P.l2 * inv);
-                    }
+                for (int m = lane; m < cnt; m += 32) {
+                    const int2 q = lds2(path_s + 8u * (unsigned)m);
+                    atomicAdd(cb + q.x, __int_as_float(q.y) * inv);
                 }
             }
             __syncwarp();
