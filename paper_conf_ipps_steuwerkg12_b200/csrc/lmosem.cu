@@ -134,13 +134,13 @@ lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
 }
 
 // Number of z-slabs for the projection: the brick image must stay L2-resident during a
-// pass (L2 126 MB; budget 48 MB per image slab leaves room for the event stream and the
+// pass (L2 126 MB; budget 56 MB per image slab leaves room for the event stream and the
 // per-event fp array). 1 = the single fused pass.
 int n_slabs(const lmosem_ctx* ctx) {
     const int max_slabs = std::max(1, ctx->dims[2] / 2);
     if (ctx->slabs_forced > 0) return std::min(ctx->slabs_forced, max_slabs);
     const double bytes = 4.0 * (double)ctx->nbf;
-    const double budget = 48.0 * 1024 * 1024;
+    const double budget = 56.0 * 1024 * 1024;
     return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
 }
 
