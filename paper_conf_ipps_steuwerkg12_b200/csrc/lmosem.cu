@@ -55,6 +55,8 @@ struct lmosem_ctx {
     cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
     int rank = 0, world = 1;
     ncclComm_t comm = nullptr;
+    bool nccl_mem = false;                          // c, fb from ncclMemAlloc (NVLS-capable)
+    void* reg_c = nullptr, * reg_fb = nullptr;       // ncclCommRegister handles
     int num_sms = 0, proj_blocks_per_sm = 0;
     bool failed = false;
     std::string err;
@@ -427,8 +429,34 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     ctx->stream = ctx->own_stream;
-    cuda(cudaMalloc(&ctx->c, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(c)");
-    cuda(cudaMalloc(&ctx->fb, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(fb)");
+    if (s != LMOSEM_OK) return bail(s);
+    if (dist) {  // a communicator whenever a dist is given (world == 1 runs the 1-rank combine)
+        ncclUniqueId id;
+        std::memcpy(&id, dist->nccl_unique_id, sizeof(id));
+        ncclResult_t r = ncclCommInitRank(&ctx->comm, world, id, rank);
+        if (r != ncclSuccess) {
+            ctx->comm = nullptr;
+            ctx->err = std::string("ncclCommInitRank: ") + ncclGetErrorString(r);
+            return bail(LMOSEM_ENCCL);
+        }
+        // the exchanged images come from ncclMemAlloc and are registered with the
+        // communicator, so NCCL can run the reduce-scatter / all-gather zero-copy (and
+        // through NVLS in-switch reduction on NVSwitch systems)
+        const size_t bytes = sizeof(float) * 8 * ctx->nb_alloc;
+        if (ncclMemAlloc((void**)&ctx->c, bytes) == ncclSuccess && ncclMemAlloc((void**)&ctx->fb, bytes) == ncclSuccess) {
+            ctx->nccl_mem = true;
+            if (ncclCommRegister(ctx->comm, ctx->c, bytes, &ctx->reg_c) != ncclSuccess) ctx->reg_c = nullptr;
+            if (ncclCommRegister(ctx->comm, ctx->fb, bytes, &ctx->reg_fb) != ncclSuccess) ctx->reg_fb = nullptr;
+        } else {
+            if (ctx->c) ncclMemFree(ctx->c);
+            if (ctx->fb) ncclMemFree(ctx->fb);
+            ctx->c = ctx->fb = nullptr;
+        }
+    }
+    if (!ctx->nccl_mem) {
+        cuda(cudaMalloc(&ctx->c, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(c)");
+        cuda(cudaMalloc(&ctx->fb, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(fb)");
+    }
     cuda(cudaMalloc(&ctx->norm, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(norm)");
     cuda(cudaMalloc(&ctx->scratch, sizeof(float) * V), "cudaMalloc(scratch)");
     cuda(cudaMalloc(&ctx->work, sizeof(unsigned long long) * kWorkSlots), "cudaMalloc(work)");
@@ -448,16 +476,6 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
     cuda(cudaStreamSynchronize(ctx->stream), "sync");
     if (s != LMOSEM_OK) return bail(s);
-    if (dist) {  // a communicator whenever a dist is given (world == 1 runs the 1-rank all-reduce)
-        ncclUniqueId id;
-        std::memcpy(&id, dist->nccl_unique_id, sizeof(id));
-        ncclResult_t r = ncclCommInitRank(&ctx->comm, world, id, rank);
-        if (r != ncclSuccess) {
-            ctx->comm = nullptr;
-            ctx->err = std::string("ncclCommInitRank: ") + ncclGetErrorString(r);
-            return bail(LMOSEM_ENCCL);
-        }
-    }
     *out = ctx;
     return LMOSEM_OK;
 }
@@ -763,6 +781,15 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (!ctx) return LMOSEM_OK;
     if (ctx->stream) cudaStreamSynchronize(ctx->stream);
     if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
+    if (ctx->comm) {
+        if (ctx->reg_c) ncclCommDeregister(ctx->comm, ctx->reg_c);
+        if (ctx->reg_fb) ncclCommDeregister(ctx->comm, ctx->reg_fb);
+    }
+    if (ctx->nccl_mem) {
+        if (ctx->c) ncclMemFree(ctx->c);
+        if (ctx->fb) ncclMemFree(ctx->fb);
+        ctx->c = ctx->fb = nullptr;
+    }
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     for (auto& pm : ctx->pending)
         for (int k = 0; k < 5; ++k) cudaEventDestroy(pm.e[k]);
