@@ -495,3 +495,29 @@ def test_reconstruct_file_matches_device(pkg, tmp_path):
     rec.subset_step(dev(ev[:cfg.n_events]), ff)
     rec.synchronize()
     rec.close()
+
+
+def test_user_stream_and_argument_errors(pkg):
+    """Work enqueued on a non-default torch stream stays ordered with torch ops on it;
+    bad offsets / iteration counts are EINVAL and leave the context usable."""
+    cfg, ev, s = inputs("C1")
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    side = torch.cuda.Stream()
+    with torch.cuda.stream(side):
+        rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), stream=side)
+        evd = torch.from_numpy(ev).cuda(non_blocking=False)
+        f = torch.ones(cfg.n_voxels, device="cuda")
+        rec.reconstruct(evd, off, 1, f)
+        f2 = f * 1.0  # torch op on the same stream, after the library's work
+    side.synchronize()
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, np.ones(cfg.n_voxels))
+    assert rel_l2(f2.cpu().numpy().astype(np.float64), ref) <= REL_L2_RECON
+    for bad_off, iters in [(off[::-1].copy(), 1), (off - 5, 1), (off, -1)]:
+        with pytest.raises(pkg.LmosemError) as e:
+            rec.reconstruct(evd, bad_off, iters, f)
+        assert e.value.status == 1
+    g0 = f.clone()
+    rec.reconstruct(evd, off, 0, f)  # zero iterations: f unchanged
+    rec.synchronize()
+    assert torch.equal(f, g0)
+    rec.close()
