@@ -53,6 +53,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-sample", type=int, default=200_000, help="events in the oracle's timed sample")
     ap.add_argument("--slabs", type=int, default=0, help="z-slab passes for step 1 (0 = automatic)")
+    ap.add_argument("--combine", default="auto", choices=["auto", "allreduce", "isd", "fused"],
+                    help="combine of the per-GPU error images for N > 1 (default: isd)")
     return ap.parse_args()
 
 
@@ -211,6 +213,8 @@ def main():
     stream = torch.cuda.current_stream()
     rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, norm, dist=pkg.make_dist(rank, world), stream=stream)
     rec.set_slabs(args.slabs)
+    if world > 1 and args.combine != "auto":
+        rec.set_combine({"allreduce": 1, "isd": 2, "fused": 3}[args.combine])  # collective
     N = cfg.n_events
 
     def subset(k):
@@ -376,7 +380,8 @@ def main():
                    "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block, f copy, c allreduce)",
                    "l2": "not flushed: inputs larger than L2 (events of the 10 subsets, 24 B x N x 10); f, c "
                          "are the reconstruction's persistent state (flushed variant: flushed_subset_step)",
-                   "z_slabs": rec.slabs},
+                   "z_slabs": rec.slabs, "combine": {0: "none", 1: "allreduce", 2: "isd", 3: "fused"}.get(
+                       rec.combine if world > 1 else 0)},
         "s_per_recon": tot_ms / K * L * 1e-3, "s_per_recon_e2e": s_recon,
         "timed_region": f"{K} subset iterations = lmosem_reconstruct calls over the {L} subsets, cycling; "
                         "CUDA events around each call on the library's stream",

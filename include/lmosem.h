@@ -120,6 +120,14 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  * 0 (default) = ISD when world > 1, else ALLREDUCE. EINVAL for other values. */
 #define LMOSEM_COMBINE_ALLREDUCE 1
 #define LMOSEM_COMBINE_ISD 2
+/* LMOSEM_COMBINE_FUSED (opt-in): the ISD switch as ONE kernel over
+ * NVLink peer memory (NCCL 2.28 symmetric windows + device communicator): rank r reads its
+ * block of c summed over ranks (multimem.ld_reduce in the NVSwitch when available, else
+ * peer loads), updates it and writes the new f block to every rank (multimem.st or peer
+ * stores), between two LSA barriers. Selecting it is COLLECTIVE (window registration); it
+ * needs a context with a dist and all ranks in one NVLink domain, else ENCCL (not fatal,
+ * the mode is unchanged). Validated on a 1-rank communicator only. */
+#define LMOSEM_COMBINE_FUSED 3
 lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode);
 
 /* The combine mode in effect (-1 for a NULL context). */

@@ -18,6 +18,7 @@
 
 #include "lmosem.h"
 #include "lmosem_kernels.cuh"
+#include "lmosem_fused.cuh"
 
 #define LMOSEM_API extern "C" __attribute__((visibility("default")))
 
@@ -57,6 +58,11 @@ struct lmosem_ctx {
     ncclComm_t comm = nullptr;
     bool nccl_mem = false;                          // c, fb from ncclMemAlloc (NVLS-capable)
     void* reg_c = nullptr, * reg_fb = nullptr;       // ncclCommRegister handles
+    // fused combine (LMOSEM_COMBINE_FUSED): symmetric windows + device communicator
+    ncclWindow_t win_c = nullptr, win_fb = nullptr;
+    ncclDevComm dev_comm{};
+    bool dev_comm_ok = false, dev_comm_mm = false;
+    int fused_ctas = 0;
     int num_sms = 0, proj_blocks_per_sm = 0;
     bool failed = false;
     std::string err;
@@ -254,7 +260,20 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
     if ((s = mark(ctx, pm, 1))) return s;
     if ((s = launch_project(ctx, ev + b, e - b, nullptr, 0))) return s;
     if ((s = mark(ctx, pm, 2))) return s;
-    if (ctx->comm && combine_mode(ctx) == LMOSEM_COMBINE_ISD) {
+    if (ctx->comm && combine_mode(ctx) == LMOSEM_COMBINE_FUSED && ctx->dev_comm_ok) {
+        // NEXT-1: reduce-scatter + update + all-gather as one kernel over peer memory
+        const int64_t chunk = ctx->nb_alloc / ctx->world;
+        if ((s = mark(ctx, pm, 3))) return s;
+        if (ctx->dev_comm_mm)
+            lmk::k_combine_fused<true><<<ctx->fused_ctas, 256, 0, ctx->stream>>>(
+                ctx->dev_comm, ctx->win_c, ctx->win_fb, ctx->norm, ctx->c, ctx->fb, chunk, ctx->bricks.nb);
+        else
+            lmk::k_combine_fused<false><<<ctx->fused_ctas, 256, 0, ctx->stream>>>(
+                ctx->dev_comm, ctx->win_c, ctx->win_fb, ctx->norm, ctx->c, ctx->fb, chunk, ctx->bricks.nb);
+        CK(cudaGetLastError());
+        ctx->st.launches++;
+        if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
+    } else if (ctx->comm && combine_mode(ctx) == LMOSEM_COMBINE_ISD) {
         // PAPER.md lines 509-518 (Listing 3 l.15-19): PSD -> ISD. Reduce-scatter c so rank r
         // holds the sum over its brick block, update only that block, all-gather f.
         const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
@@ -482,7 +501,36 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
 
 LMOSEM_API lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode) {
     USABLE(ctx);
-    if (mode < 0 || mode > LMOSEM_COMBINE_ISD) return fail(ctx, LMOSEM_EINVAL, "set_combine: bad mode");
+    if (mode < 0 || mode > LMOSEM_COMBINE_FUSED) return fail(ctx, LMOSEM_EINVAL, "set_combine: bad mode");
+    if (mode == LMOSEM_COMBINE_FUSED && !ctx->dev_comm_ok) {
+        // collective: symmetric windows over c and the brick f, and a device communicator
+        // with one LSA barrier per CTA of the fused kernel (multimem when the team has it)
+        if (!ctx->comm || !ctx->nccl_mem)
+            return LMOSEM_ENCCL;  // needs a communicator and NCCL-allocated images (not fatal)
+        CK(cudaStreamSynchronize(ctx->stream));
+        const size_t bytes = sizeof(float) * 8 * ctx->nb_alloc;
+        if (!ctx->win_c && ncclCommWindowRegister(ctx->comm, ctx->c, bytes, &ctx->win_c, NCCL_WIN_COLL_SYMMETRIC) != ncclSuccess)
+            return (ctx->win_c = nullptr, LMOSEM_ENCCL);
+        if (!ctx->win_fb && ncclCommWindowRegister(ctx->comm, ctx->fb, bytes, &ctx->win_fb, NCCL_WIN_COLL_SYMMETRIC) != ncclSuccess)
+            return (ctx->win_fb = nullptr, LMOSEM_ENCCL);
+        ctx->fused_ctas = ctx->num_sms;
+        ncclDevCommRequirements reqs;
+        std::memset(&reqs, 0, sizeof(reqs));
+        reqs.lsaBarrierCount = ctx->fused_ctas;
+        reqs.lsaMultimem = ctx->world > 1;
+        ncclResult_t r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
+        if (r != ncclSuccess && reqs.lsaMultimem) {
+            reqs.lsaMultimem = false;
+            r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
+        }
+        if (r != ncclSuccess) return LMOSEM_ENCCL;
+        if (ctx->dev_comm.lsaSize != ctx->world) {  // not one NVLink domain: keep the NCCL collectives
+            ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
+            return LMOSEM_ENCCL;
+        }
+        ctx->dev_comm_ok = true;
+        ctx->dev_comm_mm = reqs.lsaMultimem;
+    }
     ctx->combine = mode;
     return LMOSEM_OK;
 }
@@ -782,6 +830,9 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (ctx->stream) cudaStreamSynchronize(ctx->stream);
     if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
     if (ctx->comm) {
+        if (ctx->dev_comm_ok) ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
+        if (ctx->win_c) ncclCommWindowDeregister(ctx->comm, ctx->win_c);
+        if (ctx->win_fb) ncclCommWindowDeregister(ctx->comm, ctx->win_fb);
         if (ctx->reg_c) ncclCommDeregister(ctx->comm, ctx->reg_c);
         if (ctx->reg_fb) ncclCommDeregister(ctx->comm, ctx->reg_fb);
     }

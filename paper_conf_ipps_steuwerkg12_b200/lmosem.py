@@ -29,7 +29,7 @@ EXPORTS = (
     "lmosem_sensitivity", "lmosem_set_norm", "lmosem_set_combine", "lmosem_get_combine",
     "lmosem_reconstruct_file",
 )
-COMBINE_ALLREDUCE, COMBINE_ISD = 1, 2
+COMBINE_ALLREDUCE, COMBINE_ISD, COMBINE_FUSED = 1, 2, 3
 
 
 class LmosemError(RuntimeError):
@@ -276,7 +276,7 @@ class Reconstructor:
         self._check(self._lib.lmosem_update(self._h, _dev_ptr(f, "float32", self.V), _dev_ptr(c, "float32", self.V)))
 
     def set_combine(self, mode: int):
-        """0 = auto, COMBINE_ALLREDUCE or COMBINE_ISD (see lmosem.h)."""
+        """0 = auto, COMBINE_ALLREDUCE, COMBINE_ISD or COMBINE_FUSED (collective; see lmosem.h)."""
         self._check(self._lib.lmosem_set_combine(self._h, int(mode)))
 
     @property
