@@ -409,8 +409,8 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
             ctx->geom.B[k] = (int)(m[k] - M[k] / 2);
         }
     }
-    // <= 3 pieces per dominant-axis slab
-    ctx->cap = 3 * std::max(dims[0], std::max(dims[1], dims[2]));
+    // <= 3 pieces per dominant-axis slab; >= 96 entries (768 B) to stage a 32-event tile
+    ctx->cap = std::max(96, 3 * std::max(dims[0], std::max(dims[1], dims[2])));
     ctx->proj_smem = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
 
     lmosem_status s = LMOSEM_OK;

@@ -279,8 +279,8 @@ __device__ __forceinline__ float warp_sum(float v) {
     return v;
 }
 
-// Loads event idx (6 floats): three 8-byte streaming loads; consecutive lanes read
-// consecutive 24-byte records (768 contiguous bytes per warp).
+// Loads event idx (6 floats) directly: three 8-byte streaming loads (fallback for event
+// tiles that are not 16-byte aligned).
 __device__ __forceinline__ void load_event(const float* __restrict__ events, int64_t idx, float ev[6]) {
     const float2* p = reinterpret_cast<const float2*>(events + 6 * idx);
     float2 a = __ldcs(p), b = __ldcs(p + 1), c = __ldcs(p + 2);
@@ -353,12 +353,30 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
         if (base >= n) break;
         const int64_t idx = base + lane;
         const bool mine_ev = lane < batch && idx < n;
+        // event tile staging: the claimed events (24 B each, contiguous) are loaded with
+        // coalesced 16-byte vector loads into the head of the warp's path buffer (idle at
+        // this point), then each lane reads its record from shared memory
+        const int m = (int)min((int64_t)batch, n - base);
+        const float* tile_g = events + 6 * base;
+        const bool vec = ((((uintptr_t)tile_g) & 15) == 0) && ((m & 1) == 0);
+        float4* tile_s = reinterpret_cast<float4*>(smem_path + (size_t)wib * cap);
+        if (vec) {
+            const float4* src = reinterpret_cast<const float4*>(tile_g);
+            for (int q = lane; q < (3 * m) / 2; q += 32) tile_s[q] = __ldcs(src + q);
+        }
+        __syncwarp();
         Lor mine;
         bool ok = false;
         float fp_known = 1.0f;  // MODE 4 back-projects len * 1
         if (mine_ev) {
             float ev[6];
-            load_event(events, idx, ev);
+            if (vec) {
+                const float2* r = reinterpret_cast<const float2*>(tile_s) + 3 * lane;
+                const float2 a = r[0], b = r[1], c = r[2];
+                ev[0] = a.x; ev[1] = a.y; ev[2] = b.x; ev[3] = b.y; ev[4] = c.x; ev[5] = c.y;
+            } else {
+                load_event(events, idx, ev);
+            }
             ok = lor_setup(ev, g, mine);
             if (MODE == 3) {
                 fp_known = fp[idx];
@@ -366,6 +384,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const 
             }
         }
         if (MODE == 1 && mine_ev && !ok) fp[idx] = 0.0f;
+        __syncwarp();  // the tile is dead: the path buffer may be overwritten
         unsigned mask = __ballot_sync(0xffffffffu, ok);
         while (mask) {
             const int src = __ffs(mask) - 1;
