@@ -119,6 +119,17 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     const double rDa = 1.0 / Da;
     const double sb = Db * rDa, sc = Dc * rDa;
     const double fx = (double)(1LL << FIX_BITS);
+    // Guard: by the clip, the minor positions over the slab range lie in [0, n] up to
+    // rounding; coordinates so large that float64 cannot resolve the clip (|p| ~ 1e20 mm)
+    // would push them outside the 2-voxel halo (and the Q24.40 range) -> drop such LORs.
+    {
+        const double wbf = u1b + ((double)i0 - u1a) * sb, wbl = wbf + (double)(il + 1 - i0) * sb;
+        const double wcf = u1c + ((double)i0 - u1a) * sc, wcl = wcf + (double)(il + 1 - i0) * sc;
+        const double nb = (double)sel3(g.n, b), nc = (double)sel3(g.n, c);
+        if (!(fmin(wbf, wbl) > -1.0 && fmax(wbf, wbl) < nb + 1.0 && fmin(wcf, wcl) > -1.0 &&
+              fmax(wcf, wcl) < nc + 1.0))
+            return false;
+    }
     // stored frame: an axis moving up is mirrored, w' = -w - 2^-40, so every moving axis
     // moves down and its distance to the next plane is its fraction (the 2^-40 offset keeps
     // an exactly integral position inside its half-open voxel: distance = one voxel)

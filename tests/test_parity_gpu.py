@@ -526,3 +526,24 @@ def test_user_stream_and_argument_errors(pkg):
     rec.synchronize()
     assert torch.equal(f, g0)
     rec.close()
+
+
+def test_pathological_coordinates_do_not_fault(pkg):
+    """Events with coordinates float64 cannot resolve against the volume (|p| ~ 1e20-1e38
+    mm), near-coincident endpoints and subnormal separations must not fault the kernel or
+    disturb the other events' result (they contribute nothing or a valid path)."""
+    cfg, ev, s = inputs("C1")
+    good = ev[:2000]
+    big = np.float32(1e30)
+    bad = np.array([[-big, 0.3, 0.2, big, 0.3, 0.2],
+                    [-3e38, -3e38, -3e38, 3e38, 3e38, 3e38],
+                    [1e20, 1e-20, 0.0, -1e20, 2e-20, 0.1],
+                    [0.1, 0.2, 0.3, 0.1, 0.2, np.nextafter(np.float32(0.3), np.float32(1))],
+                    [-7.0, 1e-30, 0.5, 7.0, -1e-30, 0.5]], np.float32)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.subset_step(dev(np.concatenate([good, bad])), f)
+    rec.synchronize()  # would raise on an illegal address
+    got = f.cpu().numpy().astype(np.float64)
+    assert np.all(np.isfinite(got)) and np.all(got >= 0)
+    rec.close()
