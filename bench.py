@@ -53,6 +53,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-sample", type=int, default=200_000, help="events in the oracle's timed sample")
     ap.add_argument("--slabs", type=int, default=0, help="z-slab passes for step 1 (0 = automatic)")
+    ap.add_argument("--e2e-file", action="store_true",
+                    help="also time lmosem_reconstruct_file from a raw list-mode file (page cache)")
     ap.add_argument("--combine", default="auto", choices=["auto", "allreduce", "isd", "fused"],
                     help="combine of the per-GPU error images for N > 1 (default: isd)")
     return ap.parse_args()
@@ -312,6 +314,21 @@ def main():
                "note": f"lmosem_reconstruct_host over {L} subsets x {reps} (pinned host events streamed per subset, "
                        f"overlapped with projection; pinned f H2D/D2H once per reconstruction), wall clock"}
         s_recon = float(te.item()) / reps
+        if args.e2e_file:
+            import tempfile
+            with tempfile.TemporaryDirectory() as td:
+                path = os.path.join(td, f"{name}_rank{rank}.lm")
+                ev_host.tofile(path)
+                fd_ = torch.ones(cfg.n_voxels, device=dev)
+                rec.reconstruct_file(path, offs, 1, fd_)  # warm (page cache, staging buffers)
+                torch.cuda.synchronize()
+                t0 = time.perf_counter()
+                for _ in range(reps):
+                    rec.reconstruct_file(path, offs, 1, fd_)
+                tfile = time.perf_counter() - t0
+            e2e["file"] = {"value": N * L * reps / tfile, "unit": "events/s",
+                           "what": "lmosem_reconstruct_file: raw list-mode file (page cache) -> pread into pinned "
+                                   "double buffers -> H2D overlapped with projection; f on the device"}
     else:
         s_recon = None
 

@@ -65,7 +65,7 @@ def build(force: bool = False, verbose: bool = False, defines=(), out: str | Non
            "-Xcompiler", "-fPIC,-fvisibility=hidden", "-shared",
            "-I", os.path.join(ROOT, "include"), "-I", CSRC, "-I", inc,
            os.path.join(CSRC, "lmosem.cu"), "-o", tmp,
-           "-L", lib, "-l:libnccl.so.2", f"-Xlinker=-rpath={lib}"]
+           "-L", lib, "-l:libnccl.so.2", f"-Xlinker=-rpath={lib}", "-lpthread"]
     res = subprocess.run(cmd, capture_output=True, text=True)
     if res.returncode != 0:
         raise RuntimeError("nvcc failed:\n" + res.stdout + res.stderr)
