@@ -102,7 +102,9 @@ lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t
 lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
 
 /* Creates a context on the current CUDA device.
- *   dims[3]     = {nx, ny, nz} > 0, V < 2^31
+ *   dims[3]     = {nx, ny, nz} > 0, V < 2^31 (padded internal image < 2^31 floats), and
+ *                 max(nx, ny, nz) <= 1210: the per-warp path buffer (3 pieces per
+ *                 dominant-axis slab) must fit in shared memory (EINVAL otherwise)
  *   voxel_mm[3] = voxel size in mm, finite and > 0 (float64: the geometry is float64)
  *   norm        = V float32 sensitivity image s (device or host); copied, caller keeps it
  *   dist        = NULL for one GPU, else the rank/world/NCCL id (collective init;

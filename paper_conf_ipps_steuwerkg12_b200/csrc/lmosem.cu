@@ -362,6 +362,9 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         V *= dims[k];
     }
     if (V >= (int64_t(1) << 31)) return LMOSEM_EINVAL;
+    // per-warp path buffer: 8 warps x 3 pieces per slab x 8 B must fit the 227 KB opt-in
+    // shared memory of sm_100a (checked again against the device below)
+    if (std::max(dims[0], std::max(dims[1], dims[2])) > 1210) return LMOSEM_EINVAL;
     int rank = 0, world = 1;
     if (dist) {
         rank = dist->rank;
