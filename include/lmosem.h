@@ -139,7 +139,7 @@ int32_t lmosem_get_combine(const lmosem_ctx* ctx);
  * image is too large for L2 — pass A accumulates each event's forward projection over
  * slabs of the volume, pass B back-projects slab by slab with the complete fp — so each
  * launch touches one L2-sized image slab. n_slabs = 0 (default) picks the count from a
- * 56 MB-per-slab L2 budget (1 = single fused pass); n_slabs > 0 forces it (clamped to
+ * 72 MB-per-slab L2 budget (1 = single fused pass); n_slabs > 0 forces it (clamped to
  * nz/2). The result is the same up to fp32 rounding. EINVAL if n_slabs < 0. */
 lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs);
 

@@ -47,7 +47,7 @@ struct lmosem_ctx {
     float* fb = nullptr;       // brick copy of the current f
     float* norm = nullptr;     // s in bricks (halo = 0)
     float* scratch = nullptr;  // V floats, row layout (norm upload)
-    int cap = 0;               // path-piece capacity per warp
+    int cap = 0;               // path-piece capacity per warp of the full clip box (the largest launch)
     int slabs_forced = 0;      // z-slab count (0 = automatic from the L2 budget)
     float* fp_acc = nullptr;   // per-event forward projections of the z-slab passes
     unsigned long long* work = nullptr;  // k_project work counters (one per launch in a step)
@@ -64,7 +64,13 @@ struct lmosem_ctx {
     ncclDevComm dev_comm{};
     bool dev_comm_ok = false, dev_comm_mm = false;
     int fused_ctas = 0;
-    int num_sms = 0, proj_blocks_per_sm = 0;
+    int num_sms = 0;
+    struct Occ {
+        int mode;
+        size_t smem;
+        int blocks;
+    };
+    std::vector<Occ> occ;      // k_project residency per (mode, path-buffer bytes)
     bool failed = false;
     std::string err;
     // timing
@@ -142,38 +148,74 @@ lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
     return LMOSEM_OK;
 }
 
-// Number of z-slabs for the projection: the brick image must stay L2-resident during a
-// pass (L2 126 MB; budget 56 MB per image slab leaves room for the event stream and the
-// per-event fp array). 1 = the single fused pass.
+// Number of z-slabs for the projection: the brick image slab of a pass should stay
+// L2-resident (L2 126 MB; a 72 MB budget per image slab leaves room for the event stream
+// and the per-event fp array; measured at C4, 208 MB: 2/3/4/5 slabs 27.1/24.5/25.2/26.3
+// ms). 1 = the single fused pass.
 int n_slabs(const lmosem_ctx* ctx) {
     const int max_slabs = std::max(1, ctx->dims[2] / 2);
     if (ctx->slabs_forced > 0) return std::min(ctx->slabs_forced, max_slabs);
     const double bytes = 4.0 * (double)ctx->nbf;
-    const double budget = 56.0 * 1024 * 1024;
+    const double budget = 72.0 * 1024 * 1024;
     return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
 }
 
 constexpr int kWorkSlots = 1024;  // counters, reused round-robin (zeroed per launch)
 
+// Path-buffer entries per warp for one launch: the forward-only modes (1, 2) keep no path
+// and need only the 32-event tile (96 entries); the others hold <= 3 pieces per dominant-axis
+// slab of the launch's clip box (a z-slab pass: max(nx, ny, slab height)).
+int launch_cap(int mode, const lmk::GridGeom& g) {
+    if (mode == 1 || mode == 2) return 96;
+    int m = 0;
+    for (int k = 0; k < 3; ++k) m = std::max(m, g.chi[k] - g.clo[k]);
+    return std::max(96, 3 * m);
+}
+
+// Resident CTAs per SM of k_project<mode> with `smem` bytes of path buffers (cached).
+lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks) {
+    for (const auto& o : ctx->occ)
+        if (o.mode == mode && o.smem == smem) {
+            *blocks = o.blocks;
+            return LMOSEM_OK;
+        }
+    int b = 0;
+    switch (mode) {
+        case 0: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<0>, lmk::PROJ_THREADS, smem)); break;
+        case 1: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<1>, lmk::PROJ_THREADS, smem)); break;
+        case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2>, lmk::PROJ_THREADS, smem)); break;
+        case 3: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<3>, lmk::PROJ_THREADS, smem)); break;
+        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<4>, lmk::PROJ_THREADS, smem)); break;
+    }
+    b = std::max(1, b);
+    ctx->occ.push_back({mode, smem, b});
+    *blocks = b;
+    return LMOSEM_OK;
+}
+
 lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
+    const int cap = launch_cap(mode, g);
+    const size_t sm = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)cap;
+    int per_sm = 1;
+    lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm);
+    if (s) return s;
     const int64_t wpb = lmk::PROJ_THREADS / 32;
-    const int64_t resident = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm * wpb;
+    const int64_t resident = (int64_t)ctx->num_sms * per_sm * wpb;
     // events per claim: 32 when every warp gets >= 4 claims, else smaller (>= 4)
     int batch = 32;
     while (batch > 4 && n < (int64_t)batch * resident * 4) batch >>= 1;
     const int64_t blocks_needed = ((n + batch - 1) / batch + wpb - 1) / wpb;
-    const int64_t cap = (int64_t)ctx->num_sms * ctx->proj_blocks_per_sm;
-    const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, cap));
-    const size_t sm = ctx->proj_smem;
+    const int64_t max_grid = (int64_t)ctx->num_sms * per_sm;
+    const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, max_grid));
     unsigned long long* work = ctx->work + ctx->work_next;
     ctx->work_next = (ctx->work_next + 1) % kWorkSlots;
     CK(cudaMemsetAsync(work, 0, sizeof(unsigned long long), ctx->stream));
     switch (mode) {
-        case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
-        case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
-        case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
-        case 3: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
-        default: lmk::k_project<4><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, ctx->cap, work, batch); break;
+        case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 3: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        default: lmk::k_project<4><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
     }
     CK(cudaGetLastError());
     ctx->st.launches++;
@@ -445,10 +487,6 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
          "smem attr");
     cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
          "smem attr");
-    cuda(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&ctx->proj_blocks_per_sm, lmk::k_project<0>, lmk::PROJ_THREADS,
-                                                       ctx->proj_smem),
-         "occupancy");
-    if (ctx->proj_blocks_per_sm < 1) ctx->proj_blocks_per_sm = 1;
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     ctx->stream = ctx->own_stream;

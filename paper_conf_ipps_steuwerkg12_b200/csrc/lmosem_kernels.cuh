@@ -330,9 +330,16 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
+#ifndef LMK_SLAB_MIN_BLOCKS
+#define LMK_SLAB_MIN_BLOCKS LMK_MIN_BLOCKS  // CTAs per SM of the z-slab passes (modes 2, 3)
+#endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
+template <int MODE>
+constexpr int proj_min_blocks() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN_BLOCKS : LMK_MIN_BLOCKS; }
 
-// Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2.
+// Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2
+// (<= 3 per dominant-axis slab of the launch's clip box; MODEs 1/2 keep no path: only the
+// 32-event tile, 96 entries).
 // MODE 0: fused forward + back-projection into cb (step 1, image resident in L2).
 // MODE 1: forward projection only, fp[i] = fp (tests).
 // MODE 2: z-slab pass A: fp[i] += forward projection of the part of LOR i in the slab.
@@ -343,7 +350,7 @@ constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
 template <int MODE>
-__global__ void __launch_bounds__(PROJ_THREADS, LMK_MIN_BLOCKS) k_project(const float* __restrict__ events, int64_t n,
+__global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap,
                                                              unsigned long long* __restrict__ work, int batch) {

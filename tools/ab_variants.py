@@ -13,6 +13,7 @@ VARIANTS = {
     # (rejected variants are listed with their numbers in DESIGN.md §7)
     "default": [],
     "c256x2": ["LMK_MIN_BLOCKS=2"],
+    "slab4": ["LMK_SLAB_MIN_BLOCKS=4"],
 }
 
 
