@@ -318,6 +318,25 @@ def test_c4_full_size_properties(pkg):
     rec.close()
 
 
+def test_c4_full_subset_matches_oracle(pkg):
+    """configs[3] at full size, element by element: one 10^7-event subset through
+    lmosem_subset_step in the launch configuration bench.py times (automatic z-slab
+    count), against the oracle's subset step over the same events (~20 s of host work)."""
+    cfg = lmgen.CONFIGS["C4"]
+    ev = lmgen.subset_events(cfg, 1)
+    s = lmgen.norm(cfg)
+    f0 = np.random.default_rng(12).uniform(0.5, 2.0, cfg.n_voxels).astype(np.float32)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    assert rec.slabs > 1
+    f = dev(f0)
+    rec.subset_step(dev(ev), f)
+    rec.synchronize()
+    got = f.cpu().numpy().astype(np.float64)
+    rec.close()
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev, s, f0)
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
 # ------------------------------------------------------------------ z-slab (out-of-L2) form
 @pytest.mark.parametrize("slabs", [2, 3, 5])
 def test_zslab_passes_match_oracle_c1(pkg, slabs):
