@@ -221,6 +221,31 @@ def test_c1_host_reconstruct_matches_device(pkg):
     rec.close()
 
 
+@pytest.mark.parametrize("slabs", [0, 3])
+def test_c2_host_reconstruct_pipelined(pkg, slabs):
+    """C2-sized host path: the first subset's upload is chunked (projected as the chunks
+    land) and the final f is downloaded per brick z-range as the update finishes; the
+    result is the oracle's 2-subset reconstruction (rel L2) and equals the device path's."""
+    cfg = lmgen.CONFIGS["C2"]
+    L = 2
+    ev = lmgen.events(cfg, 0, cfg.n_events * L)
+    s = lmgen.norm(cfg)
+    off = np.arange(L + 1) * cfg.n_events
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    rec.set_slabs(slabs)
+    f0 = np.random.default_rng(21).uniform(0.5, 2.0, cfg.n_voxels).astype(np.float32)
+    fh = f0.copy()
+    rec.reconstruct_host(torch.from_numpy(ev).pin_memory(), off, 1, fh)
+    fd = dev(f0)
+    rec.reconstruct(dev(ev), off, 1, fd)
+    rec.synchronize()
+    rec.close()
+    assert maxrel(fh.astype(np.float64), fd.cpu().numpy().astype(np.float64)) <= 1e-5
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, f0.astype(np.float64))
+    assert rel_l2(fh.astype(np.float64), ref) <= REL_L2_RECON
+    assert maxrel(fh.astype(np.float64), ref) <= 2 * MAXREL_SUBSET
+
+
 def test_emulated_psd_ranks(pkg):
     """PAPER.md §IV.A (lines 476-485): summing the error images of the P blocks of a
     subset (each computed separately, as P ranks would) equals the whole subset's."""
