@@ -483,10 +483,13 @@ def test_combine_modes_single_rank(pkg, combine):
 
 
 @pytest.mark.parametrize("dims,vox", [((17, 12, 9), (1.0, 0.75, 1.5)), ((33, 5, 64), (0.6, 2.0, 0.45)),
-                                      ((1, 40, 7), (1.0, 1.0, 1.0))])
+                                      ((1, 40, 7), (1.0, 1.0, 1.0)),
+                                      ((1210, 6, 5), (0.25, 1.0, 1.0)), ((3, 1210, 4), (1.0, 0.2, 1.0))])
 def test_odd_extents_anisotropic_voxels(pkg, dims, vox):
     """Odd extents (padding, halo), anisotropic voxels (dominant axis in voxel units) and
-    segments that start or end inside the volume, against the oracle."""
+    segments that start or end inside the volume, against the oracle. The 1210-voxel
+    extents are the largest lmosem_init accepts: a whole-volume path buffer of
+    3 * 1210 pieces per warp fills the 227 KB of shared memory (1 CTA per SM)."""
     g = oracle.geom(dims, vox)
     V = int(np.prod(dims))
     half = 0.5 * np.asarray(dims) * np.asarray(vox)
