@@ -139,9 +139,17 @@ def l2_peak_gbs(V: int):
     return out
 
 
+def host_cores() -> int:
+    try:
+        return len(os.sched_getaffinity(0))
+    except AttributeError:  # pragma: no cover
+        return os.cpu_count() or 1
+
+
 def cpu_baseline(cfg, sample: int):
     """The float64 oracle as it stands, on this host's cores, on a bounded sample."""
     import oracle
+    oracle.set_threads(host_cores())  # all host cores (torchrun exports OMP_NUM_THREADS=1)
     ev = lmgen.subset_events(cfg, 0, sample)
     s = lmgen.norm(cfg)
     g = oracle.geom(cfg.dims, cfg.voxel_mm)
@@ -158,6 +166,7 @@ def run_reference(args, cfg, rank):
     if rank != 0:
         return
     import oracle
+    oracle.set_threads(host_cores())  # rank 0 alone runs: all host cores
     sample = min(args.cpu_sample, cfg.n_events)
     g = oracle.geom(cfg.dims, cfg.voxel_mm)
     s = lmgen.norm(cfg)
