@@ -17,6 +17,9 @@ def sector_keys(ix, iy, iz, dom, layout):
         return (ix >> 1) + 1000 * ((iy >> 1) + 1000 * (iz >> 1))
     if layout == "x-major rows of 8":
         return (ix >> 3) + 1000 * (iy + 1000 * iz)
+    if layout[0] == "abs":  # one layout for every LOR: brick extents along (x, y, z)
+        _, ex, ey, ez = layout
+        return (ix // ex) + 1000 * ((iy // ey) + 1000 * (iz // ez))
     ea, eb, ec = layout  # per-dominant-axis layouts: extents along (a, b, c)
     ax = [ix, iy, iz]
     b = 1 if dom == 0 else 0
@@ -26,11 +29,13 @@ def sector_keys(ix, iy, iz, dom, layout):
 
 def main():
     n = int(sys.argv[1]) if len(sys.argv) > 1 else 3000
-    cfg = lmgen.CONFIGS["C2"]
+    cfg = lmgen.CONFIGS[sys.argv[2] if len(sys.argv) > 2 else "C2"]
     g = oracle.geom(cfg.dims, cfg.voxel_mm)
     nx, ny, _ = cfg.dims
     ev = lmgen.subset_events(cfg, 0, n)
-    layouts = ["brick 2x2x2", "x-major rows of 8", (8, 1, 1), (4, 1, 2), (4, 2, 1)]
+    layouts = ["brick 2x2x2", "x-major rows of 8", (8, 1, 1), (4, 1, 2), (4, 2, 1),
+               ("abs", 4, 2, 1), ("abs", 2, 4, 1), ("abs", 4, 1, 2), ("abs", 1, 4, 2), ("abs", 2, 1, 4),
+               ("abs", 1, 2, 4), ("abs", 8, 1, 1), ("abs", 1, 1, 8)]
     sectors = {str(L): 0 for L in layouts}
     pieces = 0
     for e in ev:
