@@ -34,7 +34,9 @@
  *    (copy(add)): by default reduce-scatter + block update + all-gather (the paper's
  *    PSD -> ISD switch), or all-reduce + full update (lmosem_set_combine). Either way the
  *    replicas of f are identical on return.
- *  - Errors: every call returns a status. EINVAL for bad arguments (nothing enqueued);
+ *  - Errors: every call returns a status. EINVAL for bad arguments (nothing enqueued),
+ *    including a "device" buffer the GPU cannot dereference (pageable host memory;
+ *    device, managed and pinned host memory are accepted — cudaPointerGetAttributes);
  *    ECUDA/ENCCL for runtime failures (message in lmosem_last_error), after which the
  *    context answers ESTATE to everything except lmosem_last_error and lmosem_destroy.
  *  - Threading: one host thread per context; one context per GPU (rank).

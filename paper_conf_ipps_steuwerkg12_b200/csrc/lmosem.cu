@@ -103,6 +103,24 @@ lmosem_status fail(lmosem_ctx* ctx, lmosem_status s, const std::string& msg) {
     return s;
 }
 
+// A buffer the kernels may dereference: device or managed memory, or pinned host memory
+// (mapped through UVA). Pageable host memory (cudaMemoryTypeUnregistered) is rejected
+// before anything is enqueued, instead of faulting in a kernel and poisoning the context.
+bool device_accessible(const void* p) {
+    if (!p) return true;  // NULL / empty handled by the callers' own checks
+    cudaPointerAttributes a;
+    if (cudaPointerGetAttributes(&a, p) != cudaSuccess) {
+        (void)cudaGetLastError();
+        return false;
+    }
+    return a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged ||
+           (a.type == cudaMemoryTypeHost && a.devicePointer != nullptr);
+}
+
+bool device_accessible(const void* a, const void* b, const void* c = nullptr) {
+    return device_accessible(a) && device_accessible(b) && device_accessible(c);
+}
+
 #define CK(call)                                                                                    \
     do {                                                                                            \
         cudaError_t e_ = (call);                                                                    \
@@ -645,6 +663,8 @@ LMOSEM_API lmosem_status lmosem_set_stream(lmosem_ctx* ctx, void* stream) {
 LMOSEM_API lmosem_status lmosem_subset_step(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events, float* f) {
     USABLE(ctx);
     if (!f || n_events < 0 || (n_events > 0 && !events)) return fail(ctx, LMOSEM_EINVAL, "subset_step: bad arguments");
+    if (!device_accessible(f, n_events > 0 ? events : nullptr))
+        return fail(ctx, LMOSEM_EINVAL, "subset_step: events / f are not device-accessible memory");
     return subset_iteration(ctx, events, n_events, f, true, true, true);
 }
 
@@ -653,6 +673,8 @@ LMOSEM_API lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event*
     USABLE(ctx);
     if (!f || n_iterations < 0 || check_offsets(offsets, n_subsets) || (offsets[n_subsets] > offsets[0] && !events))
         return fail(ctx, LMOSEM_EINVAL, "reconstruct: bad arguments");
+    if (!device_accessible(f, offsets[n_subsets] > offsets[0] ? events : nullptr))
+        return fail(ctx, LMOSEM_EINVAL, "reconstruct: events / f are not device-accessible memory");
     const int64_t total = (int64_t)n_iterations * n_subsets;
     int64_t step = 0;
     for (int32_t it = 0; it < n_iterations; ++it)
@@ -738,6 +760,7 @@ LMOSEM_API lmosem_status lmosem_reconstruct_file(lmosem_ctx* ctx, const char* pa
     USABLE(ctx);
     if (!path || !f || n_iterations < 0 || check_offsets(offsets, n_subsets))
         return fail(ctx, LMOSEM_EINVAL, "reconstruct_file: bad arguments");
+    if (!device_accessible(f)) return fail(ctx, LMOSEM_EINVAL, "reconstruct_file: f is not device-accessible memory");
     const int fd = open(path, O_RDONLY);
     if (fd < 0) return fail(ctx, LMOSEM_EIO, std::string("reconstruct_file: open ") + path + ": " + strerror(errno));
     struct stat sb;
@@ -871,6 +894,8 @@ LMOSEM_API lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event*
     USABLE(ctx);
     if (!f || !c_out || n_events < 0 || (n_events > 0 && !events))
         return fail(ctx, LMOSEM_EINVAL, "error_image: bad arguments");
+    if (!device_accessible(f, c_out, n_events > 0 ? events : nullptr))
+        return fail(ctx, LMOSEM_EINVAL, "error_image: buffers are not device-accessible memory");
     lmosem_status s;
     if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
     if ((s = launch_project(ctx, events, n_events, nullptr, 0))) return s;
@@ -882,6 +907,8 @@ LMOSEM_API lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* eve
     USABLE(ctx);
     if (!f || n_events < 0 || (n_events > 0 && (!events || !fp_out)))
         return fail(ctx, LMOSEM_EINVAL, "forward: bad arguments");
+    if (!device_accessible(f, n_events > 0 ? events : nullptr, n_events > 0 ? fp_out : nullptr))
+        return fail(ctx, LMOSEM_EINVAL, "forward: buffers are not device-accessible memory");
     lmosem_status s;
     if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
     return launch_project(ctx, events, n_events, fp_out, 1);
@@ -892,6 +919,8 @@ LMOSEM_API lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event*
     USABLE(ctx);
     if (!s_out || n_events < 0 || (n_events > 0 && !events))
         return fail(ctx, LMOSEM_EINVAL, "sensitivity: bad arguments");
+    if (!device_accessible(s_out, n_events > 0 ? events : nullptr))
+        return fail(ctx, LMOSEM_EINVAL, "sensitivity: buffers are not device-accessible memory");
     int64_t b = 0, e = n_events;
     block_range(n_events, ctx->rank, ctx->world, &b, &e);
     lmosem_status s;
@@ -913,6 +942,7 @@ LMOSEM_API lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm) {
 LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {
     USABLE(ctx);
     if (!f || !c) return fail(ctx, LMOSEM_EINVAL, "update: bad arguments");
+    if (!device_accessible(f, c)) return fail(ctx, LMOSEM_EINVAL, "update: f / c are not device-accessible memory");
     lmosem_status s;
     if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
     if ((s = launch_to_brick(ctx, c, ctx->c))) return s;

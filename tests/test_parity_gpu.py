@@ -572,6 +572,22 @@ def test_user_stream_and_argument_errors(pkg):
     rec.reconstruct(evd, off, 0, f)  # zero iterations: f unchanged
     rec.synchronize()
     assert torch.equal(f, g0)
+    # pageable host memory passed as a device buffer through the raw C ABI: EINVAL before
+    # anything is enqueued, the context stays usable; pinned host memory is accepted (UVA)
+    lib, h = rec._lib, rec._h
+    ev_host = np.ascontiguousarray(ev[:64])
+    f_host = np.ones(cfg.n_voxels, np.float32)
+    assert lib.lmosem_subset_step(h, ev_host.ctypes.data, 64, f.data_ptr()) == 1
+    assert b"device-accessible" in lib.lmosem_last_error(h)
+    assert lib.lmosem_subset_step(h, evd.data_ptr(), 64, f_host.ctypes.data) == 1
+    assert lib.lmosem_update(h, f_host.ctypes.data, f.data_ptr()) == 1
+    ev_pinned = torch.from_numpy(ev[:64].copy()).pin_memory()
+    f3 = torch.ones(cfg.n_voxels, device="cuda")
+    f4 = torch.ones(cfg.n_voxels, device="cuda")
+    assert lib.lmosem_subset_step(h, ev_pinned.data_ptr(), 64, f3.data_ptr()) == 0
+    rec.subset_step(evd[:64], f4)
+    rec.synchronize()
+    torch.testing.assert_close(f3, f4, rtol=1e-6, atol=0)
     rec.close()
 
 
