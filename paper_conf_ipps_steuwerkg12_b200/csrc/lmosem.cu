@@ -185,6 +185,11 @@ int n_slabs(const lmosem_ctx* ctx) {
 
 constexpr int kWorkSlots = 1024;  // counters, reused round-robin (zeroed per launch)
 
+// Path-buffer entries for a clip box whose largest extent is m voxels: <= 3 pieces per
+// dominant-axis slab, >= 96 (the 32-event tile), rounded up to a multiple of 4 so every
+// warp's buffer starts 32-byte aligned (the tile is staged with 16-byte vector stores).
+int path_cap(int m) { return (std::max(96, 3 * m) + 3) & ~3; }
+
 // Path-buffer entries per warp for one launch: the forward-only modes (1, 2) keep no path
 // and need only the 32-event tile (96 entries); the others hold <= 3 pieces per dominant-axis
 // slab of the launch's clip box (a z-slab pass: max(nx, ny, slab height)).
@@ -192,7 +197,7 @@ int launch_cap(int mode, const lmk::GridGeom& g) {
     if (mode == 1 || mode == 2) return 96;
     int m = 0;
     for (int k = 0; k < 3; ++k) m = std::max(m, g.chi[k] - g.clo[k]);
-    return std::max(96, 3 * m);
+    return path_cap(m);
 }
 
 // Resident CTAs per SM of k_project<mode> with `smem` bytes of path buffers (cached).
@@ -520,8 +525,8 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
             ctx->geom.B[k] = (int)(m[k] - M[k] / 2);
         }
     }
-    // <= 3 pieces per dominant-axis slab; >= 96 entries (768 B) to stage a 32-event tile
-    ctx->cap = std::max(96, 3 * std::max(dims[0], std::max(dims[1], dims[2])));
+    // whole-volume path buffer (the largest launch; see path_cap)
+    ctx->cap = path_cap(std::max(dims[0], std::max(dims[1], dims[2])));
     ctx->proj_smem = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
 
     lmosem_status s = LMOSEM_OK;
