@@ -77,3 +77,41 @@ def test_fuzz_matches_oracle(pkg, seed):
     rel = np.abs(got[mm] - ref[mm]) / ref[mm]
     assert float(rel.max()) <= 1e-4, (dims, vox, slabs, float(rel.max()))
     assert np.array_equal(got[s == 0], f0.astype(np.float64)[s == 0])
+
+
+@pytest.mark.parametrize("seed", range(12))
+def test_fuzz_reconstruct_paths(pkg, seed, tmp_path):
+    """Random subset offsets (empty subsets included) and iteration counts through the
+    device, host and file entry points against the oracle's reconstruction; sensitivity
+    image of the same LORs against the oracle's."""
+    dims, vox, ev, s, f0, slabs = case(100 + seed)
+    rng = np.random.default_rng(seed)
+    L = int(rng.integers(1, 6))
+    cuts = np.sort(rng.integers(0, len(ev) + 1, L - 1))
+    off = np.concatenate([[0], cuts, [len(ev)]]).astype(np.int64)
+    iters = int(rng.integers(1, 3))
+    g = oracle.geom(dims, vox)
+    ref = oracle.reconstruct(g, ev, off, iters, s, f0.astype(np.float64))
+    rec = pkg.Reconstructor(dims, vox, dev(s))
+    rec.set_slabs(slabs)
+    fd = dev(f0)
+    rec.reconstruct(dev(ev), off, iters, fd)
+    fh = f0.copy()
+    rec.reconstruct_host(torch.from_numpy(ev).pin_memory(), off, iters, fh)
+    path = tmp_path / "ev.lm"
+    ev.tofile(path)
+    ff = dev(f0)
+    rec.reconstruct_file(str(path), off, iters, ff)
+    sens = torch.empty(int(np.prod(dims)), device="cuda")
+    rec.sensitivity(dev(ev), sens)
+    rec.synchronize()
+    rec.close()
+    for got in (fd.cpu().numpy(), fh, ff.cpu().numpy()):
+        got = got.astype(np.float64)
+        assert float(np.linalg.norm(got - ref) / np.linalg.norm(ref)) <= 1e-3
+        mm = ref > 1e-3 * ref.max()
+        assert float(np.max(np.abs(got[mm] - ref[mm]) / ref[mm])) <= 1e-4 * (1 + L * iters)
+    ref_s = oracle.sensitivity(g, ev)
+    got_s = sens.cpu().numpy().astype(np.float64)
+    ms = ref_s > 1e-3 * ref_s.max()
+    assert float(np.max(np.abs(got_s[ms] - ref_s[ms]) / ref_s[ms])) <= 1e-4
