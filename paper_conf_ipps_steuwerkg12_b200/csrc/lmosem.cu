@@ -499,6 +499,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         ctx->vox[k] = voxel_mm[k];
         ctx->geom.n[k] = dims[k];
         ctx->geom.lo[k] = -0.5 * (double)dims[k] * voxel_mm[k];
+        ctx->geom.v[k] = voxel_mm[k];
         ctx->geom.inv_v[k] = 1.0 / voxel_mm[k];
     }
     for (int k = 0; k < 3; ++k) {

@@ -39,6 +39,7 @@ struct GridGeom {
     int A[3], B[3];   // brick index of padded coordinate p on axis k: A[k]*p + B[k]*(p & 1)
     int clo[3], chi[3];  // clip box in voxels: [0, n) except z = [zlo, zhi) of a z-slab pass
     double lo[3];     // volume lower corner (mm): -n*v/2
+    double v[3];      // voxel size (mm)
     double inv_v[3];  // 1 / voxel size (1/mm)
 };
 
@@ -85,7 +86,10 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
         double p2 = (double)ev[3 + k];
         ok = ok && isfinite(p1[k]) && isfinite(p2);
         d[k] = p2 - p1[k];
-        u1[k] = (p1[k] - g.lo[k]) * g.inv_v[k];
+        // voxel coordinate by division: a stationary axis' voxel row (a LOR lying in or
+        // near a voxel face) is then decided exactly as the oracle decides it,
+        // floor((p - lo) / v) in float64 (reading S6)
+        u1[k] = (p1[k] - g.lo[k]) / g.v[k];
         D[k] = d[k] * g.inv_v[k];
     }
     if (!ok) return false;
@@ -100,8 +104,8 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
             double t0 = (lo - u1[k]) * r, t1 = (hi - u1[k]) * r;
             amin = fmax(amin, fmin(t0, t1));
             amax = fmin(amax, fmax(t0, t1));
-        } else if (u1[k] < lo || u1[k] >= hi) {
-            return false;
+        } else if (u1[k] < lo || u1[k] >= hi || p1[k] < g.lo[k] || p1[k] >= g.lo[k] + (double)g.n[k] * g.v[k]) {
+            return false;  // parallel to axis k and outside (the volume test in mm as the oracle's)
         }
     }
     if (!(amax > amin)) return false;
@@ -134,8 +138,15 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     // moves down and its distance to the next plane is its fraction (the 2^-40 offset keeps
     // an exactly integral position inside its half-open voxel: distance = one voxel)
     {
-        const long long wb = __double2ll_rn((u1b + ((double)i0 - u1a) * sb) * fx);
-        const long long wc = __double2ll_rn((u1c + ((double)i0 - u1a) * sc) * fx);
+        // floor decided in float64, fraction rounded to Q.40 below 1: a stationary axis
+        // (s = 0: w = u1 exactly) keeps the oracle's voxel row
+        auto fix = [fx](double u) {
+            const double fl = floor(u);
+            const long long q = min(__double2ll_rn((u - fl) * fx), (1LL << FIX_BITS) - 1);
+            return (long long)fl * (1LL << FIX_BITS) + q;
+        };
+        const long long wb = fix(u1b + ((double)i0 - u1a) * sb);
+        const long long wc = fix(u1c + ((double)i0 - u1a) * sc);
         const long long qb = __double2ll_rn(sb * fx), qc = __double2ll_rn(sc * fx);
         L.wb0 = sb > 0.0 ? -wb - 1 : wb;
         L.sb = sb > 0.0 ? -qb : qb;

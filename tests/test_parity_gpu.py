@@ -610,3 +610,42 @@ def test_pathological_coordinates_do_not_fault(pkg):
     got = f.cpu().numpy().astype(np.float64)
     assert np.all(np.isfinite(got)) and np.all(got >= 0)
     rec.close()
+
+
+@pytest.mark.parametrize("vox", [(0.3, 0.7, 1.1), (0.45, 1.3, 0.9), (1.0, 1.0, 1.0)])
+def test_lors_in_voxel_faces(pkg, vox):
+    """Axis-parallel LORs lying exactly in voxel faces (float32 coordinates nearest to the
+    planes lo + k*v, as crystal grids produce): the voxel row is a floating-point decision,
+    taken by both sides as floor((p - lo) / v) in float64 (reading S6: the voxel above the
+    face; a face that rounds to the upper outer face is outside)."""
+    dims = (20, 16, 12)
+    g = oracle.geom(dims, vox)
+    lo = -0.5 * np.asarray(dims) * np.asarray(vox)
+    rng = np.random.default_rng(7)
+    ev = []
+    for i in range(600):
+        a = i % 3
+        b, c = (a + 1) % 3, (a + 2) % 3
+        p = np.zeros(3)
+        p[b] = lo[b] + rng.integers(0, dims[b] + 1) * vox[b]  # a face (or the outer faces)
+        p[c] = lo[c] + rng.integers(0, dims[c] + 1) * vox[c] if i % 2 else rng.uniform(lo[c], -lo[c])
+        q = p.copy()
+        p[a], q[a] = lo[a] - 3.0, -lo[a] + 3.0
+        ev.append(np.concatenate([p, q]))
+    ev = np.array(ev, np.float32)
+    s = np.ones(int(np.prod(dims)), np.float32)
+    f0 = rng.uniform(0.5, 2.0, int(np.prod(dims))).astype(np.float32)
+    rec = pkg.Reconstructor(dims, vox, dev(s))
+    fp = torch.empty(len(ev), device="cuda")
+    rec.forward(dev(ev), dev(f0), fp)
+    f = dev(f0)
+    rec.subset_step(dev(ev), f)
+    rec.synchronize()
+    rec.close()
+    ref_fp = oracle.forward(g, ev, f0)
+    got_fp = fp.cpu().numpy().astype(np.float64)
+    assert np.array_equal(got_fp > 0, ref_fp > 0)
+    m = ref_fp > 0
+    assert np.max(np.abs(got_fp[m] - ref_fp[m]) / ref_fp[m]) <= 2e-6
+    ref = oracle.subset_step(g, ev, s, f0)
+    assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
