@@ -115,3 +115,41 @@ def test_fuzz_reconstruct_paths(pkg, seed, tmp_path):
     got_s = sens.cpu().numpy().astype(np.float64)
     ms = ref_s > 1e-3 * ref_s.max()
     assert float(np.max(np.abs(got_s[ms] - ref_s[ms]) / ref_s[ms])) <= 1e-4
+
+
+@pytest.mark.parametrize("scale", [1e-3, 1e3])
+@pytest.mark.parametrize("seed", range(4))
+def test_fuzz_scaled_and_short(pkg, seed, scale):
+    """The same geometry in other units (voxel sizes 1e-3 and 1e3 times larger) and very
+    short segments (1e-3 to 1 voxel, both endpoints inside, often inside one voxel)."""
+    dims, vox, ev, s, f0, slabs = case(200 + seed)
+    rng = np.random.default_rng(300 + seed)
+    vox = tuple(v * scale for v in vox)
+    ev = ev.astype(np.float64) * scale
+    half = 0.5 * np.asarray(dims) * np.asarray(vox)
+    k = len(ev) // 3  # a third of the LORs replaced by short interior segments
+    c = rng.uniform(-0.95 * half, 0.95 * half, (k, 3))
+    d = rng.normal(size=(k, 3))
+    d /= np.linalg.norm(d, axis=1, keepdims=True)
+    ln = rng.uniform(1e-3, 1.0, (k, 1)) * min(vox)
+    ev[:k] = np.concatenate([c - 0.5 * ln * d, c + 0.5 * ln * d], axis=1)
+    ev = ev.astype(np.float32)
+    g = oracle.geom(dims, vox)
+    rec = pkg.Reconstructor(dims, vox, dev(s))
+    rec.set_slabs(slabs)
+    fp = torch.empty(len(ev), device="cuda")
+    rec.forward(dev(ev), dev(f0), fp)
+    f = dev(f0)
+    rec.subset_step(dev(ev), f)
+    rec.synchronize()
+    rec.close()
+    ref_fp = oracle.forward(g, ev, f0)
+    got_fp = fp.cpu().numpy().astype(np.float64)
+    m = ref_fp > 0
+    assert np.array_equal(got_fp > 0, m)
+    err = np.abs(got_fp[m] - ref_fp[m])
+    assert np.all(err <= 2e-6 * ref_fp[m] + 1e-6 * max(vox)), float(np.max(err / ref_fp[m]))
+    ref = oracle.subset_step(g, ev, s, f0)
+    got = f.cpu().numpy().astype(np.float64)
+    mm = ref > 1e-3 * ref.max()
+    assert float(np.max(np.abs(got[mm] - ref[mm]) / ref[mm])) <= 1e-4
