@@ -341,6 +341,9 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
+#ifndef LMK_GUIDED_DIV
+#define LMK_GUIDED_DIV 2  // guided claims: remaining / (LMK_GUIDED_DIV * warps); 0 = fixed claims
+#endif
 #ifndef LMK_SLAB_MIN_BLOCKS
 #define LMK_SLAB_MIN_BLOCKS LMK_MIN_BLOCKS  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
@@ -372,20 +375,32 @@ __global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_proje
     const int wib = threadIdx.x >> 5;
     const unsigned path_s = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)wib * cap);
     const unsigned lt = (1u << lane) - 1u;
-    // dynamic work distribution: each warp claims `batch` (<= 32) consecutive events at a
-    // time from a global counter (zeroed before the launch), so unequal LOR lengths and
-    // small per-rank subsets do not leave a tail of idle warps
+    // dynamic work distribution: each warp claims consecutive events from a global counter
+    // (zeroed before the launch), so unequal LOR lengths and small per-rank subsets do not
+    // leave idle warps. Guided claim sizes: `batch` (<= 32) while there is plenty of work,
+    // then remaining / (LMK_GUIDED_DIV * warps in the grid), even and >= 2 (claims stay
+    // 16-byte aligned) — a 32-event claim takes a warp ~0.1 ms at C2, so fixed claims
+    // left a tail of that length at the end of every launch
+    const int64_t warps_in_grid = (int64_t)gridDim.x * (blockDim.x >> 5);
+    int take = batch;
     for (;;) {
         unsigned long long claim = 0;
-        if (lane == 0) claim = atomicAdd(work, (unsigned long long)batch);
+        if (lane == 0) claim = atomicAdd(work, (unsigned long long)take);
         const int64_t base = (int64_t)__shfl_sync(0xffffffffu, claim, 0);
         if (base >= n) break;
         const int64_t idx = base + lane;
-        const bool mine_ev = lane < batch && idx < n;
+        const bool mine_ev = lane < take && idx < n;
         // event tile staging: the claimed events (24 B each, contiguous) are loaded with
         // coalesced 16-byte vector loads into the head of the warp's path buffer (idle at
         // this point), then each lane reads its record from shared memory
-        const int m = (int)min((int64_t)batch, n - base);
+        const int m = (int)min((int64_t)take, n - base);
+#if LMK_GUIDED_DIV > 0
+        {
+            const int64_t rem = n - base - take;  // work left after this claim (estimate)
+            const int64_t g = rem / (LMK_GUIDED_DIV * warps_in_grid);
+            take = batch <= 2 ? batch : (int)max((int64_t)2, min((int64_t)batch, g)) & ~1;
+        }
+#endif
         const float* tile_g = events + 6 * base;
         const bool vec = ((((uintptr_t)tile_g) & 15) == 0) && ((m & 1) == 0);
         float4* tile_s = reinterpret_cast<float4*>(smem_path + (size_t)wib * cap);

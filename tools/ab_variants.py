@@ -14,6 +14,9 @@ VARIANTS = {
     "default": [],
     "c256x2": ["LMK_MIN_BLOCKS=2"],
     "slab4": ["LMK_SLAB_MIN_BLOCKS=4"],
+    "guided1": ["LMK_GUIDED_DIV=1"],
+    "guided4": ["LMK_GUIDED_DIV=4"],
+    "fixed": ["LMK_GUIDED_DIV=0"],
 }
 
 
