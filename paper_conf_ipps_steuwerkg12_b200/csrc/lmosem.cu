@@ -548,16 +548,17 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
 
 
-    cuda(cudaFuncSetAttribute(lmk::k_project<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
-         "smem attr");
-    cuda(cudaFuncSetAttribute(lmk::k_project<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
-         "smem attr");
-    cuda(cudaFuncSetAttribute(lmk::k_project<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
-         "smem attr");
-    cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
-         "smem attr");
-    cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ctx->proj_smem),
-         "smem attr");
+    // The limit is a per-function, process-wide attribute: set it to the device maximum
+    // (not this context's need), so a smaller context created later cannot lower it under
+    // a larger one (each launch passes its own size).
+    {
+        const int smax = (int)prop.sharedMemPerBlockOptin;
+        cuda(cudaFuncSetAttribute(lmk::k_project<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+    }
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     ctx->stream = ctx->own_stream;

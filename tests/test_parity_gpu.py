@@ -649,3 +649,27 @@ def test_lors_in_voxel_faces(pkg, vox):
     assert np.max(np.abs(got_fp[m] - ref_fp[m]) / ref_fp[m]) <= 2e-6
     ref = oracle.subset_step(g, ev, s, f0)
     assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
+
+
+def test_contexts_of_different_sizes_coexist(pkg):
+    """Two contexts in one process, the small one created after the large one: each keeps
+    working (the kernels' shared-memory limits are per function, process-wide) and their
+    interleaved subsets give the same results as alone."""
+    big, evb, sb = inputs("C1")
+    cfg2 = lmgen.CONFIGS["C2"]
+    ev2 = lmgen.subset_events(cfg2, 0, 20000)
+    s2 = lmgen.norm(cfg2)
+    rec_l = pkg.Reconstructor(cfg2.dims, cfg2.voxel_mm, dev(s2))
+    rec_s = pkg.Reconstructor(big.dims, big.voxel_mm, dev(sb))
+    fl = dev(np.ones(cfg2.n_voxels, np.float32))
+    fs = dev(np.ones(big.n_voxels, np.float32))
+    rec_l.subset_step(dev(ev2), fl)
+    rec_s.subset_step(dev(evb[:big.n_events]), fs)
+    rec_l.synchronize()
+    rec_s.synchronize()
+    ref_l = oracle.subset_step(oracle.geom(cfg2.dims, cfg2.voxel_mm), ev2, s2, np.ones(cfg2.n_voxels))
+    ref_s = oracle.subset_step(oracle.geom(big.dims, big.voxel_mm), evb[:big.n_events], sb, np.ones(big.n_voxels))
+    assert maxrel(fl.cpu().numpy().astype(np.float64), ref_l) <= MAXREL_SUBSET
+    assert maxrel(fs.cpu().numpy().astype(np.float64), ref_s) <= MAXREL_SUBSET
+    rec_l.close()
+    rec_s.close()
