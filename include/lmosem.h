@@ -37,8 +37,11 @@
  *  - Errors: every call returns a status. EINVAL for bad arguments (nothing enqueued),
  *    including a "device" buffer the GPU cannot dereference (pageable host memory;
  *    device, managed and pinned host memory are accepted — cudaPointerGetAttributes);
- *    ECUDA/ENCCL for runtime failures (message in lmosem_last_error), after which the
- *    context answers ESTATE to everything except lmosem_last_error and lmosem_destroy.
+ *    ENOMEM when a call cannot allocate its working memory (the z-slab forward-projection
+ *    array, host-path staging buffers): the call has not changed f or the context's images
+ *    and the context stays usable; ECUDA/ENCCL for runtime failures (message in
+ *    lmosem_last_error), after which the context answers ESTATE to everything except
+ *    lmosem_last_error and lmosem_destroy.
  *  - Threading: one host thread per context; one context per GPU (rank).
  */
 #ifndef LMOSEM_H

@@ -128,6 +128,19 @@ bool device_accessible(const void* a, const void* b, const void* c = nullptr) {
             return fail(ctx, LMOSEM_ECUDA, std::string(#call) + ": " + cudaGetErrorString(e_));     \
     } while (0)
 
+// Allocations: out of memory is ENOMEM and leaves the context usable (the allocation error
+// is not sticky and nothing of the failed call has touched c); other errors are ECUDA.
+#define CKA(call)                                                                                   \
+    do {                                                                                            \
+        cudaError_t e_ = (call);                                                                    \
+        if (e_ == cudaErrorMemoryAllocation) {                                                      \
+            (void)cudaGetLastError();                                                               \
+            return fail(ctx, LMOSEM_ENOMEM, std::string(#call) + ": " + cudaGetErrorString(e_));   \
+        }                                                                                           \
+        if (e_ != cudaSuccess)                                                                      \
+            return fail(ctx, LMOSEM_ECUDA, std::string(#call) + ": " + cudaGetErrorString(e_));     \
+    } while (0)
+
 #define NK(call)                                                                                    \
     do {                                                                                            \
         ncclResult_t r_ = (call);                                                                   \
@@ -276,7 +289,7 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         if (ctx->fp_acc) CK(cudaFree(ctx->fp_acc));
         ctx->fp_acc = nullptr;
         ctx->fp_cap = 0;
-        CK(cudaMalloc(&ctx->fp_acc, sizeof(float) * n));
+        CKA(cudaMalloc(&ctx->fp_acc, sizeof(float) * n));
         ctx->fp_cap = n;
     }
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
@@ -709,7 +722,7 @@ lmosem_status ensure_stream_buffers(lmosem_ctx* ctx, const int64_t* offsets, int
             ctx->dev_ev[k] = nullptr;
         }
         ctx->dev_ev_cap = 0;
-        for (int k = 0; k < 2; ++k) CK(cudaMalloc(&ctx->dev_ev[k], sizeof(lmosem_event) * cap));
+        for (int k = 0; k < 2; ++k) CKA(cudaMalloc(&ctx->dev_ev[k], sizeof(lmosem_event) * cap));
         ctx->dev_ev_cap = cap;
     }
     if (pinned && cap > ctx->pin_cap) {
@@ -718,7 +731,7 @@ lmosem_status ensure_stream_buffers(lmosem_ctx* ctx, const int64_t* offsets, int
             ctx->pin_ev[k] = nullptr;
         }
         ctx->pin_cap = 0;
-        for (int k = 0; k < 2; ++k) CK(cudaHostAlloc(&ctx->pin_ev[k], sizeof(lmosem_event) * cap, cudaHostAllocDefault));
+        for (int k = 0; k < 2; ++k) CKA(cudaHostAlloc(&ctx->pin_ev[k], sizeof(lmosem_event) * cap, cudaHostAllocDefault));
         ctx->pin_cap = cap;
     }
     return LMOSEM_OK;
@@ -833,7 +846,7 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
     // this rank's block of every subset: the only events it uploads (block distribution)
     lmosem_status s0 = ensure_stream_buffers(ctx, offsets, n_subsets, false);
     if (s0) return s0;
-    if (!ctx->dev_f) CK(cudaMalloc(&ctx->dev_f, sizeof(float) * ctx->V));
+    if (!ctx->dev_f) CKA(cudaMalloc(&ctx->dev_f, sizeof(float) * ctx->V));
     // f goes up first on the copy stream (the first projection needs it), then the first
     // subset's events in kPipe chunks that the projection consumes as they land
     CK(cudaEventRecord(ctx->ev_pipe[kPipe], ctx->stream));

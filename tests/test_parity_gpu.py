@@ -673,3 +673,54 @@ def test_contexts_of_different_sizes_coexist(pkg):
     assert maxrel(fs.cpu().numpy().astype(np.float64), ref_s) <= MAXREL_SUBSET
     rec_l.close()
     rec_s.close()
+
+
+def test_out_of_memory_is_enomem_and_recoverable(pkg):
+    """A subset too large for the z-slab forward-projection array (4 B per event): ENOMEM,
+    f untouched, the context keeps working; a context failure (ECUDA) makes every later
+    call answer ESTATE (checked in a subprocess: a kernel fault poisons the CUDA context)."""
+    cfg, ev, s = inputs("C1")
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    rec.set_slabs(2)
+    evd = dev(ev[:cfg.n_events])
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    st = rec._lib.lmosem_subset_step(rec._h, evd.data_ptr(), 1 << 42, f.data_ptr())  # 16 TB fp array
+    assert st == 2, rec._lib.lmosem_last_error(rec._h)
+    rec.synchronize()
+    assert torch.all(f == 1.0).item()
+    rec.subset_step(evd, f)
+    rec.synchronize()
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], s, np.ones(cfg.n_voxels))
+    assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
+    rec.close()
+
+
+ESTATE_SCRIPT = r"""
+import ctypes, numpy as np, torch
+import paper_conf_ipps_steuwerkg12_b200 as pkg
+rec = pkg.Reconstructor((16, 16, 16), (1, 1, 1), torch.ones(4096, device="cuda"))
+lib, h = rec._lib, rec._h
+f = torch.ones(4096, device="cuda")
+ev = torch.zeros(64, 6, device="cuda")
+st1 = lib.lmosem_subset_step(h, ev.data_ptr(), 1 << 30, f.data_ptr())  # reads far past the buffer
+st2 = lib.lmosem_synchronize(h)
+st3 = lib.lmosem_subset_step(h, ev.data_ptr(), 64, f.data_ptr())
+print(st1, st2, st3, lib.lmosem_last_error(h).decode()[:60])
+print("destroy", lib.lmosem_destroy(h))
+"""
+
+
+def test_runtime_failure_poisons_context():
+    """ECUDA (a kernel reading past the caller's event buffer) -> ESTATE afterwards."""
+    import subprocess
+    import sys
+    if not torch.cuda.is_available():
+        pytest.skip("needs a GPU")
+    from conftest import ROOT
+    out = subprocess.run([sys.executable, "-c", ESTATE_SCRIPT], capture_output=True, text=True, timeout=300,
+                         cwd=ROOT)
+    lines = out.stdout.strip().splitlines()
+    assert lines, out.stderr[-2000:]
+    st1, st2, st3 = (int(x) for x in lines[0].split()[:3])
+    assert st1 == 0 and st2 == 3 and st3 == 5, lines
+    assert lines[-1] == "destroy 0"
