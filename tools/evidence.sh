@@ -14,3 +14,10 @@ python -m torch.distributed.run --nnodes 1 --nproc-per-node 1 --master-addr 127.
 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file $O/launches.csv \
     python bench.py --steps 5 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
 python -c "import __graft_entry__ as g; g.smoke(); print('smoke ok')" > $O/smoke.txt 2>&1
+# ncu --set full of the C2 projection (traffic for bench.py), C5, and the update kernel
+ncu --set full --clock-control none --import-source on -k regex:k_project -s 3 -c 1 -o $O/k_project_C2 \
+    python bench.py --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
+ncu --set full --clock-control none --import-source on -k regex:k_project -s 3 -c 1 -o $O/k_project_C5 \
+    python bench.py --config C5 --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
+ncu --set full --clock-control none -k regex:k_update -s 3 -c 1 -o $O/k_update_C2 \
+    python bench.py --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
