@@ -737,6 +737,12 @@ lmosem_status ensure_stream_buffers(lmosem_ctx* ctx, const int64_t* offsets, int
     return LMOSEM_OK;
 }
 
+#ifndef LMOSEM_READ_THREADS
+// reader threads of reconstruct_file; measured at C2 (16-core host, file in the page
+// cache): 1/2/3/4/6/8/16 threads -> 3.7/6.0/7.7/8.3-8.7/8.2/7.3/7.3e8 events/s
+#define LMOSEM_READ_THREADS 4
+#endif
+
 // Reads exactly `bytes` at `off` (retries short reads and EINTR).
 bool pread_all(int fd, void* dst, size_t bytes, off_t off) {
     char* p = static_cast<char*>(dst);
@@ -751,13 +757,13 @@ bool pread_all(int fd, void* dst, size_t bytes, off_t off) {
     return true;
 }
 
-// pread_all over up to 8 threads in contiguous 1 MiB-aligned parts (page-cache reads are
+// pread_all over up to LMOSEM_READ_THREADS threads in contiguous 1 MiB-aligned parts (page-cache reads are
 // memcpy-bound per core; one thread reads ~8 GB/s, a 24 MB subset block then takes longer
 // than its projection).
 bool pread_parallel(int fd, void* dst, size_t bytes, off_t off) {
     const size_t min_part = size_t(1) << 20;
     const unsigned hw = std::max(1u, std::thread::hardware_concurrency());
-    const size_t nt = std::min<size_t>(std::min<size_t>(8, hw), std::max<size_t>(1, bytes / min_part));
+    const size_t nt = std::min<size_t>(std::min<size_t>(LMOSEM_READ_THREADS, hw), std::max<size_t>(1, bytes / min_part));
     if (nt <= 1) return pread_all(fd, dst, bytes, off);
     std::vector<std::thread> th;
     std::vector<char> ok(nt, 1);

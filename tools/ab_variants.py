@@ -17,6 +17,12 @@ VARIANTS = {
     "guided1": ["LMK_GUIDED_DIV=1"],
     "guided4": ["LMK_GUIDED_DIV=4"],
     "fixed": ["LMK_GUIDED_DIV=0"],
+    "read1": ["LMOSEM_READ_THREADS=1"],
+    "read2": ["LMOSEM_READ_THREADS=2"],
+    "read3": ["LMOSEM_READ_THREADS=3"],
+    "read4": ["LMOSEM_READ_THREADS=4"],
+    "read6": ["LMOSEM_READ_THREADS=6"],
+    "read16": ["LMOSEM_READ_THREADS=16"],
 }
 
 
