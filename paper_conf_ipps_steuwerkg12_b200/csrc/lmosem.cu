@@ -196,7 +196,9 @@ int n_slabs(const lmosem_ctx* ctx) {
     return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
 }
 
-constexpr int kWorkSlots = 1024;  // counters, reused round-robin (zeroed per launch)
+// k_project work counters: {claimed events, exited warps} per slot, zeroed once at init;
+// the last warp out of a launch re-zeroes its slot, so no memset precedes a launch
+constexpr int kWorkSlots = 64;
 
 // Path-buffer entries for a clip box whose largest extent is m voxels: <= 3 pieces per
 // dominant-axis slab, >= 96 (the 32-event tile), rounded up to a multiple of 4 so every
@@ -248,9 +250,8 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     const int64_t blocks_needed = ((n + batch - 1) / batch + wpb - 1) / wpb;
     const int64_t max_grid = (int64_t)ctx->num_sms * per_sm;
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, max_grid));
-    unsigned long long* work = ctx->work + ctx->work_next;
+    unsigned long long* work = ctx->work + 2 * ctx->work_next;
     ctx->work_next = (ctx->work_next + 1) % kWorkSlots;
-    CK(cudaMemsetAsync(work, 0, sizeof(unsigned long long), ctx->stream));
     switch (mode) {
         case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
         case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
@@ -605,7 +606,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
     cuda(cudaMalloc(&ctx->norm, sizeof(float) * 8 * ctx->nb_alloc), "cudaMalloc(norm)");
     cuda(cudaMalloc(&ctx->scratch, sizeof(float) * V), "cudaMalloc(scratch)");
-    cuda(cudaMalloc(&ctx->work, sizeof(unsigned long long) * kWorkSlots), "cudaMalloc(work)");
+    cuda(cudaMalloc(&ctx->work, sizeof(unsigned long long) * 2 * kWorkSlots), "cudaMalloc(work)");
     for (int k = 0; k < 2; ++k) {
         cuda(cudaEventCreateWithFlags(&ctx->ev_copied[k], cudaEventDisableTiming), "cudaEventCreate");
         cuda(cudaEventCreateWithFlags(&ctx->ev_consumed[k], cudaEventDisableTiming), "cudaEventCreate");
@@ -616,6 +617,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset c");
     cuda(cudaMemsetAsync(ctx->fb, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset fb");
     cuda(cudaMemsetAsync(ctx->norm, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset norm");
+    cuda(cudaMemsetAsync(ctx->work, 0, sizeof(unsigned long long) * 2 * kWorkSlots, ctx->stream), "memset work");
     if (s == LMOSEM_OK) {
         lmk::k_row_to_brick<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->scratch, ctx->norm,
                                                                                      ctx->geom, ctx->bricks);

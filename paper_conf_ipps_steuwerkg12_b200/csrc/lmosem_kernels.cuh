@@ -376,7 +376,7 @@ __global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_proje
     const unsigned path_s = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)wib * cap);
     const unsigned lt = (1u << lane) - 1u;
     // dynamic work distribution: each warp claims consecutive events from a global counter
-    // (zeroed before the launch), so unequal LOR lengths and small per-rank subsets do not
+    // (work[0]; zero at launch), so unequal LOR lengths and small per-rank subsets do not
     // leave idle warps. Guided claim sizes: `batch` (<= 32) while there is plenty of work,
     // then remaining / (LMK_GUIDED_DIV * warps in the grid), even and >= 2 (claims stay
     // 16-byte aligned) — a 32-event claim takes a warp ~0.1 ms at C2, so fixed claims
@@ -387,7 +387,15 @@ __global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_proje
         unsigned long long claim = 0;
         if (lane == 0) claim = atomicAdd(work, (unsigned long long)take);
         const int64_t base = (int64_t)__shfl_sync(0xffffffffu, claim, 0);
-        if (base >= n) break;
+        if (base >= n) {
+            // the last warp out re-zeroes the slot for the next launch (every other warp's
+            // final claim returned before its exit count)
+            if (lane == 0 && atomicAdd(work + 1, 1ull) == (unsigned long long)warps_in_grid - 1) {
+                work[0] = 0;
+                work[1] = 0;
+            }
+            break;
+        }
         const int64_t idx = base + lane;
         const bool mine_ev = lane < take && idx < n;
         // event tile staging: the claimed events (24 B each, contiguous) are loaded with
