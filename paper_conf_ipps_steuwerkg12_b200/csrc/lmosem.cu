@@ -196,6 +196,16 @@ int n_slabs(const lmosem_ctx* ctx) {
     return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
 }
 
+#ifndef LMOSEM_STATIC_BATCH
+#define LMOSEM_STATIC_BATCH 1  // first claim size from the launch's events per warp
+#endif
+#ifndef LMOSEM_MIN_BATCH
+#define LMOSEM_MIN_BATCH 4
+#endif
+#ifndef LMOSEM_CLAIMS
+#define LMOSEM_CLAIMS 4  // target claims per warp
+#endif
+
 // k_project work counters: {claimed events, exited warps} per slot, zeroed once at init;
 // the last warp out of a launch re-zeroes its slot, so no memset precedes a launch
 constexpr int kWorkSlots = 64;
@@ -244,9 +254,11 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     if (s) return s;
     const int64_t wpb = lmk::PROJ_THREADS / 32;
     const int64_t resident = (int64_t)ctx->num_sms * per_sm * wpb;
-    // events per claim: 32 when every warp gets >= 4 claims, else smaller (>= 4)
+    // events per claim: 32 when every warp gets >= 4 claims, else smaller (>= 4); the
+    // kernel shrinks its claims further towards the end of the launch (guided)
     int batch = 32;
-    while (batch > 4 && n < (int64_t)batch * resident * 4) batch >>= 1;
+    while (LMOSEM_STATIC_BATCH && batch > LMOSEM_MIN_BATCH && n < (int64_t)batch * resident * LMOSEM_CLAIMS)
+        batch >>= 1;
     const int64_t blocks_needed = ((n + batch - 1) / batch + wpb - 1) / wpb;
     const int64_t max_grid = (int64_t)ctx->num_sms * per_sm;
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, max_grid));

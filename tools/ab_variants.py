@@ -17,6 +17,10 @@ VARIANTS = {
     "guided1": ["LMK_GUIDED_DIV=1"],
     "guided4": ["LMK_GUIDED_DIV=4"],
     "fixed": ["LMK_GUIDED_DIV=0"],
+    "nostatic": ["LMOSEM_STATIC_BATCH=0"],
+    "min2": ["LMOSEM_MIN_BATCH=2"],
+    "claims8": ["LMOSEM_CLAIMS=8", "LMOSEM_MIN_BATCH=2"],
+    "claims2": ["LMOSEM_CLAIMS=2"],
     "read1": ["LMOSEM_READ_THREADS=1"],
     "read2": ["LMOSEM_READ_THREADS=2"],
     "read3": ["LMOSEM_READ_THREADS=3"],
