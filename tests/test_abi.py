@@ -119,3 +119,19 @@ def test_product_does_not_import_oracle():
             if fn.endswith((".py", ".cu", ".cuh", ".h", ".cpp")):
                 txt = open(os.path.join(dp, fn)).read()
                 assert not re.search(r"^\s*(import|from)\s+oracle\b|liboracle|oracle\.h|oracle_\w+\(", txt, re.M), fn
+
+
+def test_l2peak_exports_and_rejects_bad_arguments(lib):
+    """include/l2peak.h (the roofline microbenchmarks): libl2peak.so exports l2peak_run
+    and rejects bad arguments with -1 before touching CUDA."""
+    txt = re.sub(r"/\*.*?\*/", "", open(os.path.join(ROOT, "include", "l2peak.h")).read(), flags=re.S)
+    decl = sorted(set(re.findall(r"\b(l2peak_\w+)\s*\(", txt)))
+    so = os.path.join(os.path.dirname(L.SO_PATH), "libl2peak.so")
+    out = os.popen(f"nm -D --defined-only {so}").read()
+    assert set(re.findall(r"\bT (l2peak_\w+)", out)) == set(decl) == {"l2peak_run"}
+    l2 = ctypes.CDLL(so)
+    l2.l2peak_run.argtypes = [ctypes.c_int, ctypes.c_int64, ctypes.c_int32, ctypes.POINTER(ctypes.c_float),
+                              ctypes.POINTER(ctypes.c_double)]
+    ms, ops = ctypes.c_float(), ctypes.c_double()
+    for mode, n, k in [(6, 1 << 20, 4), (-1, 1 << 20, 4), (0, 10, 4), (0, 1 << 20, 0), (0, 1 << 33, 4)]:
+        assert l2.l2peak_run(mode, n, k, ctypes.byref(ms), ctypes.byref(ops)) == -1
