@@ -1,13 +1,13 @@
 #!/usr/bin/env python
 """Offline layout analysis: unique 32-byte sectors per 32-piece instruction,
 path order, for C2 paths under candidate image layouts. Uses the oracle's paths (analysis
-tooling, not product code). Usage: python tools/sector_sim.py [n_events]"""
+tooling, not product code). Lives under tests/ because it runs the oracle (test infrastructure). Usage: python tests/analysis/sector_sim.py [n_events] [config]"""
 import os
 import sys
 
 import numpy as np
 
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__)))))
 import lmgen  # noqa: E402
 import oracle  # noqa: E402
 
