@@ -122,7 +122,7 @@ def measured_peaks():
         return {"hbm_gbs": 6650.0}, "fallback"
 
 
-def l2_peak_gbs(V: int):
+def l2_peak_gbs(V: int, nbf: int):
     """Live microbenchmark of random fp32 gather+RED pairs on a V-float buffer (the
     projection's L2 access mix); returns (pair ops/s, GB/s at 8 B per pair)."""
     import ctypes
@@ -136,6 +136,11 @@ def l2_peak_gbs(V: int):
         if lib.l2peak_run(mode, V, 256, ctypes.byref(ms), ctypes.byref(ops)) != 0:
             return None
         out[name] = ops.value / (ms.value * 1e-3)
+    # the update's pattern (read 3 arrays, write 2, float4) over 3 arrays of nbf floats
+    # each, 20 passes: elements/s (x 20 B = the streaming rate the update can reach)
+    ms, ops = ctypes.c_float(), ctypes.c_double()
+    if lib.l2peak_run(6, nbf, 20, ctypes.byref(ms), ctypes.byref(ops)) == 0:
+        out["stream5_elems"] = ops.value / (ms.value * 1e-3)
     return out
 
 
@@ -352,7 +357,8 @@ def main():
     ev_per_launch = N / world
     pairs = ev_per_launch * mean_path
     proj_avg_s = proj_ms / K * 1e-3
-    l2 = l2_peak_gbs(cfg.n_voxels)
+    nbf = 8 * ((cfg.dims[0] + 5) // 2) * ((cfg.dims[1] + 5) // 2) * ((cfg.dims[2] + 5) // 2)  # padded bricks
+    l2 = l2_peak_gbs(cfg.n_voxels, nbf)
     alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0  # 4 B gather + 4 B RED per path element, 24 B/event
     traffic, sectors = None, None
     try:
@@ -392,9 +398,18 @@ def main():
     hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0) / proj_avg_s / 1e9, "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
     hbm["frac"] = hbm["achieved"] / hbm["peak"]
-    upd_bytes = 24.0 * cfg.n_voxels  # read f, c, s; write f (bricks), c; write f (caller layout)
-    upd = {"bound": "hbm", "achieved": upd_bytes / (upd_ms / K * 1e-3) / 1e9, "peak": peaks["hbm_gbs"],
-           "unit": "GB/s", "peak_kind": peak_kind, "what": "k_update (24 B/voxel)"}
+    # k_update per step: read fb, c, s and write fb, c over the padded brick image (20 B per
+    # voxel); the caller's f (4 B per voxel) is written once per reconstruction (1/L steps)
+    upd_bytes = 20.0 * nbf + 4.0 * cfg.n_voxels / L
+    upd = {"achieved": upd_bytes / (upd_ms / K * 1e-3) / 1e9, "unit": "GB/s",
+           "what": f"k_update (20 B per padded voxel, {nbf} voxels, + the caller's f once per reconstruction)"}
+    if l2 and "stream5_elems" in l2 and 12.0 * nbf < 100e6:
+        # fb, c, s (12 B per voxel) stay L2-resident between projection and update
+        upd.update({"bound": "l2", "peak": l2["stream5_elems"] * 20.0 / 1e9,
+                    "peak_kind": "measured live: the update's read-3/write-2 float4 pattern streamed over three "
+                                 "L2-resident nbf-float arrays (libl2peak.so, STREAM5)"})
+    else:
+        upd.update({"bound": "hbm", "peak": peaks["hbm_gbs"], "peak_kind": peak_kind})
     upd["frac"] = upd["achieved"] / upd["peak"]
 
     line = {

@@ -17,12 +17,14 @@ enum {
     L2PEAK_PAIR_RANDOM = 2,   /* one gather + one red per op (the projection's mix) */
     L2PEAK_RED_RUN8 = 3,      /* red where each 8 lanes hit 8 consecutive floats */
     L2PEAK_PAIR_RUN8 = 4,     /* gather + red, 8-lane runs */
-    L2PEAK_PAIR_WARP32 = 5    /* gather + red, each warp on 32 consecutive floats (fully
+    L2PEAK_PAIR_WARP32 = 5,   /* gather + red, each warp on 32 consecutive floats (fully
                                  coalesced: the L2 peak for this op mix) */
+    L2PEAK_STREAM5 = 6        /* the update kernel's pattern streamed: read 3 arrays, write 2
+                                 (float4, 20 B per element); ops = elements x passes */
 };
 
-/* Runs `mode` on the current device over a buffer of n_floats floats (device memory
- * allocated and freed inside), ops_per_thread per thread on a full-occupancy grid, after
+/* Runs `mode` on the current device over a buffer of n_floats floats (three for
+ * STREAM5; device memory allocated and freed inside), ops_per_thread per thread on a full-occupancy grid, after
  * one warm-up launch. Writes the kernel time (ms, CUDA events) and the number of 4-byte
  * element operations (a pair counts as one op). Returns 0, or -1 on a CUDA error. */
 int l2peak_run(int mode, int64_t n_floats, int32_t ops_per_thread, float* ms, double* ops);

@@ -40,6 +40,21 @@ __global__ void __launch_bounds__(256) k_l2(float* __restrict__ buf, const float
     if (acc == 12345.678f) sink[0] = acc;  // keeps the gathers alive
 }
 
+// STREAM5: the update kernel's access pattern, streamed: read a, b, c, write a, b (float4),
+// a grid-stride pass over n floats per array, `ops` passes (the arrays stay L2-resident
+// when 3 * 4 * n bytes fit).
+__global__ void __launch_bounds__(256) k_stream5(float4* __restrict__ a, float4* __restrict__ b,
+                                                 const float4* __restrict__ c, uint32_t n4, int ops) {
+    for (int it = 0; it < ops; ++it)
+        for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < n4; i += gridDim.x * blockDim.x) {
+            float4 x = a[i], y = b[i];
+            const float4 z = c[i];
+            x.x = x.x * y.x + z.x; x.y = x.y * y.y + z.y; x.z = x.z * y.z + z.z; x.w = x.w * y.w + z.w;
+            a[i] = x;
+            b[i] = make_float4(0.f, 0.f, 0.f, 0.f);
+        }
+}
+
 template <int MODE>
 cudaError_t launch(float* buf, const float* src, uint32_t n, int ops, float* sink, int grid) {
     k_l2<MODE><<<grid, 256>>>(buf, src, n, ops, sink);
@@ -54,6 +69,10 @@ cudaError_t launch_mode(int mode, float* buf, const float* src, uint32_t n, int 
         case L2PEAK_RED_RUN8: return launch<L2PEAK_RED_RUN8>(buf, src, n, ops, sink, grid);
         case L2PEAK_PAIR_RUN8: return launch<L2PEAK_PAIR_RUN8>(buf, src, n, ops, sink, grid);
         case L2PEAK_PAIR_WARP32: return launch<L2PEAK_PAIR_WARP32>(buf, src, n, ops, sink, grid);
+        case L2PEAK_STREAM5:
+            k_stream5<<<grid, 256>>>(reinterpret_cast<float4*>(buf), const_cast<float4*>(reinterpret_cast<const float4*>(src)),
+                                     reinterpret_cast<const float4*>(sink), n / 4, ops);
+            return cudaGetLastError();
     }
     return cudaErrorInvalidValue;
 }
@@ -61,7 +80,7 @@ cudaError_t launch_mode(int mode, float* buf, const float* src, uint32_t n, int 
 }  // namespace
 
 L2PEAK_API int l2peak_run(int mode, int64_t n_floats, int32_t ops_per_thread, float* ms, double* ops) {
-    if (mode < 0 || mode > 5 || n_floats < 64 || n_floats >= (int64_t(1) << 32) || ops_per_thread <= 0 || !ms || !ops)
+    if (mode < 0 || mode > 6 || n_floats < 64 || n_floats >= (int64_t(1) << 32) || ops_per_thread <= 0 || !ms || !ops)
         return -1;
     int dev = 0, sms = 0, per_sm = 0;
     if (cudaGetDevice(&dev) != cudaSuccess) return -1;
@@ -74,7 +93,8 @@ L2PEAK_API int l2peak_run(int mode, int64_t n_floats, int32_t ops_per_thread, fl
     int rc = -1;
     if (cudaMalloc(&buf, sizeof(float) * n_floats) != cudaSuccess) goto done;
     if (cudaMalloc(&src, sizeof(float) * n_floats) != cudaSuccess) goto done;
-    if (cudaMalloc(&sink, sizeof(float)) != cudaSuccess) goto done;
+    if (cudaMalloc(&sink, sizeof(float) * (mode == L2PEAK_STREAM5 ? n_floats : 1)) != cudaSuccess) goto done;
+    if (mode == L2PEAK_STREAM5) cudaMemset(sink, 0, sizeof(float) * n_floats);
     cudaMemset(buf, 0, sizeof(float) * n_floats);
     cudaMemset(src, 0, sizeof(float) * n_floats);
     cudaEventCreate(&e0);
@@ -85,7 +105,7 @@ L2PEAK_API int l2peak_run(int mode, int64_t n_floats, int32_t ops_per_thread, fl
     cudaEventRecord(e1);
     if (cudaEventSynchronize(e1) != cudaSuccess) goto done;
     cudaEventElapsedTime(ms, e0, e1);
-    *ops = (double)grid * 256.0 * ops_per_thread;
+    *ops = mode == L2PEAK_STREAM5 ? (double)(n_floats / 4 * 4) * ops_per_thread : (double)grid * 256.0 * ops_per_thread;
     rc = 0;
 done:
     if (e0) cudaEventDestroy(e0);

@@ -17,7 +17,7 @@ def main():
     rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, s)
     f = torch.ones(cfg.n_voxels, device="cuda")
     out = {}
-    for P in (1, 2, 4, 8, 16):
+    for P in (1, 2, 4, 8, 16, 100, 1000):
         n = cfg.n_events // P
         off = np.array([0, n], np.int64)
         for _ in range(3):
