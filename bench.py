@@ -6,8 +6,11 @@ paper's 150x150x280 shape; s/recon).
 
 A step is one subset iteration (fused projection, c all-reduce when N > 1, update) of
 one 10^6-event subset; steps cycle through the config's 10 subsets. Inputs (events,
-norm, f) are resident in HBM before the timed region. L2 is flushed (a 256 MB write)
-before every timed step, outside the step's CUDA events. Rank 0 prints ONE JSON line.
+norm, f) are resident in HBM before the timed region. The timed region is not flushed: the
+events of the 10 subsets (240 MB at C2) exceed the 126 MB L2, f and c are the
+reconstruction's persistent state; a second measurement flushes L2 (a 256 MB write)
+before every step, outside the step's CUDA events (`flushed_subset_step`). Rank 0 prints
+ONE JSON line.
 N > 1 is launched by torchrun (one process per GPU, NCCL).
 
 --impl reference times the float64 CPU oracle (the only reference this paper-only
@@ -36,6 +39,15 @@ METRIC = "LM-OSEM events/s per subset (150x150x280)"
 # (tools/path_stats.py, oracle on a 20k-event sample)
 MEAN_PATH = {"C1": 25.37, "C2": 252.19, "C3": 252.19, "C4": 506.79, "C5": 440.96}
 FLUSH_BYTES = 256 << 20
+# The paper's own runtimes, as context only (Fig. 4b):
+# the bar heights did not survive text extraction
+PAPER_CONTEXT = {
+    "what": "average runtime of one LM-OSEM subset iteration (~10^6 events, 150x150x280), SkelCL / OpenCL / CUDA "
+            "on 1, 2 and 4 GPUs of a Tesla S1070 (GT200, 2009)",
+    "value": "bar heights not recoverable; axis 0-4 s, so <= 4 s per subset on each bar",
+    "relations": "CUDA about 20 % faster than OpenCL and SkelCL; SkelCL < 5 % overhead vs OpenCL",
+    "cite": "PAPER.md lines 586-610, 655-675 (Fig. 4b)",
+}
 
 
 def env_int(k, d):
@@ -418,7 +430,7 @@ def main():
         "dtype": "f32", "geometry_dtype": "f64", "data": "synthetic",
         "config": {"workload": f"{name}: {cfg.note} LM-OSEM {cfg.dims[0]}x{cfg.dims[1]}x{cfg.dims[2]} @ "
                                f"{cfg.voxel_mm[0]} mm, {L} subsets x {N} events, 1 iteration",
-                   "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block, f copy, c allreduce)",
+                   "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block-distributed, f copy-distributed, c combined over NCCL)",
                    "l2": "not flushed: inputs larger than L2 (events of the 10 subsets, 24 B x N x 10); f, c "
                          "are the reconstruction's persistent state (flushed variant: flushed_subset_step)",
                    "z_slabs": rec.slabs, "combine": {0: "none", 1: "allreduce", 2: "isd", 3: "fused"}.get(
@@ -432,6 +444,7 @@ def main():
         "gpu_launches": launches, "flushed_subset_step": flushed,
         "clocks": clk.summary(), "wall_s_timed_region": t_wall,
         "e2e": e2e,
+        "paper_context": PAPER_CONTEXT,
     }
     if not args.no_cpu_baseline and world == 1:
         line["cpu_baseline"] = cpu_baseline(cfg, min(args.cpu_sample, N))
