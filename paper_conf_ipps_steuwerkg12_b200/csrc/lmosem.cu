@@ -472,6 +472,19 @@ lmosem_status resolve_timing(lmosem_ctx* ctx) {
 
 }  // namespace
 
+#if LMK_TRACE
+// diagnostic builds only (not declared in lmosem.h): the per-warp timeline of the last
+// k_project launch (5 x uint64 per warp, see lmosem_kernels.cuh) to host memory, and reset
+LMOSEM_API int lmosem_debug_trace(void* out, size_t bytes) {
+    return cudaMemcpyFromSymbol(out, lmk::g_trace, std::min(bytes, sizeof(lmk::g_trace))) == cudaSuccess ? 0 : -1;
+}
+LMOSEM_API int lmosem_debug_trace_reset(void) {
+    void* p = nullptr;
+    if (cudaGetSymbolAddress(&p, lmk::g_trace) != cudaSuccess) return -1;
+    return cudaMemset(p, 0, sizeof(lmk::g_trace)) == cudaSuccess ? 0 : -1;
+}
+#endif
+
 LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.4 sm_100a"; }
 
 LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end) {

@@ -348,6 +348,19 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #define LMK_SLAB_MIN_BLOCKS LMK_MIN_BLOCKS  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
+#ifndef LMK_TRACE
+#define LMK_TRACE 0  // diagnostic builds only (tools/trace_tail.py): per-warp timeline
+#endif
+#if LMK_TRACE
+constexpr int kTraceWarps = 16384;
+// per warp: globaltimer at entry, at its first LOR, at exit; LORs processed; claims
+__device__ unsigned long long g_trace[kTraceWarps * 5];
+__device__ __forceinline__ unsigned long long gtimer() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+    return t;
+}
+#endif
 template <int MODE>
 constexpr int proj_min_blocks() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN_BLOCKS : LMK_MIN_BLOCKS; }
 
@@ -383,6 +396,10 @@ __global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_proje
     // left a tail of that length at the end of every launch
     const int64_t warps_in_grid = (int64_t)gridDim.x * (blockDim.x >> 5);
     int take = batch;
+#if LMK_TRACE
+    const int gw = blockIdx.x * (blockDim.x >> 5) + wib;
+    unsigned long long tr_start = gtimer(), tr_first = 0, tr_lors = 0, tr_claims = 0;
+#endif
     for (;;) {
         unsigned long long claim = 0;
         if (lane == 0) claim = atomicAdd(work, (unsigned long long)take);
@@ -394,6 +411,12 @@ __global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_proje
                 work[0] = 0;
                 work[1] = 0;
             }
+#if LMK_TRACE
+            if (lane == 0 && gw < kTraceWarps) {
+                unsigned long long* t = g_trace + 5 * gw;
+                t[0] = tr_start; t[1] = tr_first; t[2] = gtimer(); t[3] = tr_lors; t[4] = tr_claims;
+            }
+#endif
             break;
         }
         const int64_t idx = base + lane;
@@ -438,6 +461,11 @@ __global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_proje
         if (MODE == 1 && mine_ev && !ok) fp[idx] = 0.0f;
         __syncwarp();  // the tile is dead: the path buffer may be overwritten
         unsigned mask = __ballot_sync(0xffffffffu, ok);
+#if LMK_TRACE
+        tr_claims++;
+        if (!tr_first && mask) tr_first = gtimer();
+        tr_lors += __popc(mask);
+#endif
         while (mask) {
             const int src = __ffs(mask) - 1;
             mask &= mask - 1;
