@@ -12,7 +12,7 @@ import numpy as np
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
-OUT = os.path.join(ROOT, "variants", "liblmosem_trace.so")
+OUT = os.environ.get("LMOSEM_TRACE_LIB") or os.path.join(ROOT, "variants", "liblmosem_trace.so")
 
 
 def build():
