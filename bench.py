@@ -263,7 +263,7 @@ def main():
             a.record(stream)
             rec.reconstruct(ev[offs[l]:offs[l + m]], o, 1, f)
             b.record(stream)
-            calls.append((a, b))
+            calls.append((a, b, m))
             k0 += m
             count -= m
         return calls
@@ -289,7 +289,11 @@ def main():
         t_wall = time.perf_counter() - t_wall
     st = rec.stats()
     rec.set_timing(False)
-    tot_ms = sum(a.elapsed_time(b) for a, b in calls)
+    per_call = [(a.elapsed_time(b), m) for a, b, m in calls]
+    tot_ms = sum(t for t, _ in per_call)
+    # per-subset time of each lmosem_reconstruct call (the paper reports the average per
+    # subset; SURVEY.md §8(d) asks for the median beside it)
+    med_ms = statistics.median(t / m for t, m in per_call)
     t = torch.tensor([tot_ms, st["convert_ms"], st["project_ms"], st["combine_ms"], st["update_ms"]], device=dev,
                      dtype=torch.float64)
     if world > 1:
@@ -327,18 +331,24 @@ def main():
         reps = max(1, K // L)
         if world > 1:
             dist.barrier()
+        rec.set_timing(True)  # copy-stream CUDA events around the event uploads (h2d_ms)
         t0 = time.perf_counter()
         for _ in range(reps):
             rec.reconstruct_host(pinned, offs, 1, fh)
         te = torch.tensor([time.perf_counter() - t0], dtype=torch.float64, device=dev)
+        h2d_ms = rec.stats()["h2d_ms"]
+        rec.set_timing(False)
         if world > 1:
             dist.all_reduce(te, op=dist.ReduceOp.MAX)
         b, e = pkg.block_range(N, rank, world)
         e2e = {"value": N * L * reps / float(te.item()), "unit": "events/s",
                "h2d_bytes_per_step": int(24 * (e - b) + 4 * cfg.n_voxels / L),
                "d2h_bytes_per_step": int(4 * cfg.n_voxels / L),
+               "h2d_events_ms_per_subset": h2d_ms / (L * reps),
                "note": f"lmosem_reconstruct_host over {L} subsets x {reps} (pinned host events streamed per subset, "
-                       f"overlapped with projection; pinned f H2D/D2H once per reconstruction), wall clock"}
+                       f"overlapped with projection; pinned f H2D/D2H once per reconstruction), wall clock; "
+                       f"h2d_events_ms_per_subset = the event uploads on the copy stream (the paper's phase 1), "
+                       f"mostly hidden under the projection"}
         s_recon = float(te.item()) / reps
         if args.e2e_file:
             import tempfile
@@ -426,7 +436,7 @@ def main():
 
     line = {
         "metric": METRIC, "value": value, "unit": "events/s", "n_gpus": world, "steps": K, "warmup": args.warmup,
-        "ms_per_step": tot_ms / K, "higher_is_better": True, "scaling": "strong", "vs_baseline": None,
+        "ms_per_step": tot_ms / K, "ms_per_step_median": med_ms, "higher_is_better": True, "scaling": "strong", "vs_baseline": None,
         "dtype": "f32", "geometry_dtype": "f64", "data": "synthetic",
         "config": {"workload": f"{name}: {cfg.note} LM-OSEM {cfg.dims[0]}x{cfg.dims[1]}x{cfg.dims[2]} @ "
                                f"{cfg.voxel_mm[0]} mm, {L} subsets x {N} events, 1 iteration",
@@ -437,7 +447,8 @@ def main():
                        rec.combine if world > 1 else 0)},
         "s_per_recon": tot_ms / K * L * 1e-3, "s_per_recon_e2e": s_recon,
         "timed_region": f"{K} subset iterations = lmosem_reconstruct calls over the {L} subsets, cycling; "
-                        "CUDA events around each call on the library's stream",
+                        "CUDA events around each call on the library's stream; ms_per_step_median = median over the calls of "
+                        "their per-subset time",
         "phase_ms_per_step": {"convert_f": conv_ms / K, "project": proj_ms / K, "combine": comb_ms / K,
                               "update": upd_ms / K},
         "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_hbm_events": hbm, "roofline_update": upd,
