@@ -4,7 +4,7 @@
 # command and smoke(). Output: gpurun_out/ev/ (copied to profiles/ by hand).
 O=gpurun_out/ev
 mkdir -p $O
-python -m pytest tests -m gpu -q -s 2>&1 | grep -E "parity|passed|failed|Error" > $O/parity.txt
+(echo "# pytest -m gpu -v -s (one B200): per-test parity errors vs the float64 oracle"; python -m pytest tests -m gpu -v -s -p no:cacheprovider 2>&1 | grep -E "parity|PASSED|FAILED|passed|failed|Error") > $O/parity.txt
 python bench.py > $O/bench_C2.json 2> $O/bench_C2.err
 python bench.py --config C5 > $O/bench_C5.json 2> /dev/null
 python bench.py --config C4 --steps 20 > $O/bench_C4.json 2> /dev/null
