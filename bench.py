@@ -321,6 +321,26 @@ def main():
                "what": "lmosem_subset_step per step (incl. the f -> brick conversion), 256 MB L2 flush before each "
                        "step outside its CUDA events"}
 
+    # ---- per-rank share of a subset (N > 1 strong scaling: rank r projects N/P events of
+    # every subset): the projection of the first N/P events of subset 0 on this GPU
+    shares = None
+    if world == 1:
+        shares = {}
+        for P in (2, 4, 8):
+            n_p = N // P
+            o = np.array([0, n_p], np.int64)
+            rec.reconstruct(ev[:n_p], o, 1, f)
+            rec.set_timing(True)
+            for _ in range(10):
+                rec.reconstruct(ev[:n_p], o, 1, f)
+            stp = rec.stats()
+            rec.set_timing(False)
+            ms_p = stp["project_ms"] / stp["timed_subsets"]
+            shares[str(P)] = {"events": n_p, "project_ms": ms_p, "update_ms": stp["update_ms"] / stp["timed_subsets"],
+                              "projection_efficiency": (proj_ms / K / P) / ms_p}
+        shares["what"] = ("projection of 1/P of a subset (the per-rank step-1 work at P GPUs), CUDA events on the "
+                          "library stream; projection_efficiency = (full-subset projection / P) / this")
+
     # ---- e2e through the public API with HOST buffers: one host reconstruction over the
     # K subsets (pinned events streamed per subset, f uploaded and downloaded)
     e2e = None
@@ -452,7 +472,7 @@ def main():
         "phase_ms_per_step": {"convert_f": conv_ms / K, "project": proj_ms / K, "combine": comb_ms / K,
                               "update": upd_ms / K},
         "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_hbm_events": hbm, "roofline_update": upd,
-        "gpu_launches": launches, "flushed_subset_step": flushed,
+        "gpu_launches": launches, "flushed_subset_step": flushed, "per_rank_share": shares,
         "clocks": clk.summary(), "wall_s_timed_region": t_wall,
         "e2e": e2e,
         "paper_context": PAPER_CONTEXT,
