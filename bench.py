@@ -274,9 +274,13 @@ def main():
     # ---- timed region: K subset iterations of the reconstruction loop (lmosem_reconstruct
     # over the 10 subsets, cycling). L2 is not flushed: the events of the 10 subsets
     # (240 MB at C2) exceed the 126 MB L2; f and c are the algorithm's persistent state.
+    # The library's per-phase CUDA events are OFF here (recording them between the kernels
+    # costs ~14 us of GPU gaps per subset); an instrumented pass of the same loop right
+    # after, inside the same clock-sampled window, gives the phase times and the
+    # projection kernel's duration for the roofline.
     K = args.steps
+    K2 = min(K, 50)
     launches0 = rec.stats()["launches"]
-    rec.set_timing(True)
     if world > 1:
         dist.barrier()
     torch.cuda.synchronize()
@@ -287,8 +291,13 @@ def main():
         if world > 1:
             dist.barrier()
         t_wall = time.perf_counter() - t_wall
-    st = rec.stats()
-    rec.set_timing(False)
+        launches = int(rec.stats()["launches"] - launches0)
+        rec.set_timing(True)
+        calls2 = run_subsets(args.warmup + K, K2)
+        torch.cuda.synchronize()
+        st = rec.stats()
+        rec.set_timing(False)
+    instr_ms = sum(a.elapsed_time(b) for a, b, _ in calls2) / K2
     per_call = [(a.elapsed_time(b), m) for a, b, m in calls]
     tot_ms = sum(t for t, _ in per_call)
     # per-subset time of each lmosem_reconstruct call (the paper reports the average per
@@ -300,7 +309,8 @@ def main():
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
     tot_ms, conv_ms, proj_ms, comb_ms, upd_ms = (float(x) for x in t.tolist())
     value = N * K / (tot_ms * 1e-3)  # events of the whole job (each subset's N split over ranks)
-    launches = int(st["launches"] - launches0)
+    # phase sums below are over the K2 instrumented steps
+    conv_ms, proj_ms, comb_ms, upd_ms = (x / K2 for x in (conv_ms, proj_ms, comb_ms, upd_ms))
 
     # ---- secondary: single subset_step calls with L2 flushed before each (cold images)
     Kf = min(K, 20)
@@ -337,7 +347,7 @@ def main():
             rec.set_timing(False)
             ms_p = stp["project_ms"] / stp["timed_subsets"]
             shares[str(P)] = {"events": n_p, "project_ms": ms_p, "update_ms": stp["update_ms"] / stp["timed_subsets"],
-                              "projection_efficiency": (proj_ms / K / P) / ms_p}
+                              "projection_efficiency": (proj_ms / P) / ms_p}
         shares["what"] = ("projection of 1/P of a subset (the per-rank step-1 work at P GPUs), CUDA events on the "
                           "library stream; projection_efficiency = (full-subset projection / P) / this")
 
@@ -398,7 +408,7 @@ def main():
     mean_path = MEAN_PATH[name]
     ev_per_launch = N / world
     pairs = ev_per_launch * mean_path
-    proj_avg_s = proj_ms / K * 1e-3
+    proj_avg_s = proj_ms * 1e-3
     nbf = 8 * ((cfg.dims[0] + 5) // 2) * ((cfg.dims[1] + 5) // 2) * ((cfg.dims[2] + 5) // 2)  # padded bricks
     l2 = l2_peak_gbs(cfg.n_voxels, nbf)
     alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0  # 4 B gather + 4 B RED per path element, 24 B/event
@@ -443,7 +453,7 @@ def main():
     # k_update per step: read fb, c, s and write fb, c over the padded brick image (20 B per
     # voxel); the caller's f (4 B per voxel) is written once per reconstruction (1/L steps)
     upd_bytes = 20.0 * nbf + 4.0 * cfg.n_voxels / L
-    upd = {"achieved": upd_bytes / (upd_ms / K * 1e-3) / 1e9, "unit": "GB/s",
+    upd = {"achieved": upd_bytes / (upd_ms * 1e-3) / 1e9, "unit": "GB/s",
            "what": f"k_update (20 B per padded voxel, {nbf} voxels, + the caller's f once per reconstruction)"}
     if l2 and "stream5_elems" in l2 and 12.0 * nbf < 100e6:
         # fb, c, s (12 B per voxel) stay L2-resident between projection and update
@@ -469,8 +479,10 @@ def main():
         "timed_region": f"{K} subset iterations = lmosem_reconstruct calls over the {L} subsets, cycling; "
                         "CUDA events around each call on the library's stream; ms_per_step_median = median over the calls of "
                         "their per-subset time",
-        "phase_ms_per_step": {"convert_f": conv_ms / K, "project": proj_ms / K, "combine": comb_ms / K,
-                              "update": upd_ms / K},
+        "phase_ms_per_step": {"convert_f": conv_ms, "project": proj_ms, "combine": comb_ms, "update": upd_ms,
+                              "steps": K2, "ms_per_step_instrumented": instr_ms,
+                              "what": "library CUDA events around each phase on its stream, in an instrumented pass "
+                                      "of the same loop right after the timed region"},
         "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_hbm_events": hbm, "roofline_update": upd,
         "gpu_launches": launches, "flushed_subset_step": flushed, "per_rank_share": shares,
         "clocks": clk.summary(), "wall_s_timed_region": t_wall,
