@@ -312,12 +312,15 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
     return LMOSEM_OK;
 }
 
-// step 2 on the bricks; f_row (caller layout) is written when non-null
-lmosem_status launch_update(lmosem_ctx* ctx, float* f_row, int64_t b_begin = 0, int64_t b_end = -1) {
+// step 2 on the bricks [b_begin, b_end); f_row (caller layout) is written when non-null;
+// zero_to > 0 also re-zeroes c on every other brick of [0, zero_to) (ISD combine)
+lmosem_status launch_update(lmosem_ctx* ctx, float* f_row, int64_t b_begin = 0, int64_t b_end = -1,
+                            int64_t zero_to = 0) {
     if (b_end < 0) b_end = ctx->bricks.nb;
-    if (b_end <= b_begin) return LMOSEM_OK;
-    lmk::k_update<<<grid_for(ctx, b_end - b_begin), 256, 0, ctx->stream>>>(ctx->fb, ctx->c, ctx->norm, f_row, ctx->geom,
-                                                                           ctx->bricks, b_begin, b_end);
+    const int64_t items = zero_to > 0 ? zero_to : b_end - b_begin;
+    if (items <= 0) return LMOSEM_OK;
+    lmk::k_update<<<grid_for(ctx, items), 256, 0, ctx->stream>>>(ctx->fb, ctx->c, ctx->norm, f_row, ctx->geom,
+                                                                 ctx->bricks, b_begin, b_end, zero_to);
     CK(cudaGetLastError());
     ctx->st.launches++;
     return LMOSEM_OK;
@@ -401,10 +404,8 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         float* my_c = ctx->c + 8 * b0;
         NK(ncclReduceScatter(ctx->c, my_c, (size_t)(8 * chunk), ncclFloat32, ncclSum, ctx->comm, ctx->stream));
         if ((s = mark(ctx, pm, 3))) return s;
-        if ((s = launch_update(ctx, nullptr, b0, std::min(b0 + chunk, ctx->bricks.nb)))) return s;  // zeroes own c
-        if (b0 > 0) CK(cudaMemsetAsync(ctx->c, 0, sizeof(float) * 8 * b0, ctx->stream));
-        const int64_t rest = ctx->nb_alloc - (b0 + chunk);
-        if (rest > 0) CK(cudaMemsetAsync(my_c + 8 * chunk, 0, sizeof(float) * 8 * rest, ctx->stream));
+        // one launch: the block update (re-zeroes its c) and c <- 0 on every other brick
+        if ((s = launch_update(ctx, nullptr, b0, std::min(b0 + chunk, ctx->bricks.nb), ctx->nb_alloc))) return s;
         NK(ncclAllGather(ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk), ncclFloat32, ctx->comm, ctx->stream));
         if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
     } else {

@@ -578,13 +578,22 @@ __device__ __forceinline__ float upd1(float f, float c, float s) {
 }
 
 // Bricks [b_begin, b_end) (the whole image, or this rank's block in the ISD combine).
+// zero_to > 0 (ISD): the bricks of [0, zero_to) outside the block only get c <- 0 (the
+// reduce-scatter left this rank's partial sums there), in the same launch.
 __global__ void __launch_bounds__(256) k_update(float* __restrict__ fb, float* __restrict__ cb,
                                                 const float* __restrict__ sb, float* __restrict__ f_row, GridGeom g,
-                                                BrickIt it, int64_t b_begin, int64_t b_end) {
-    for (int64_t b = b_begin + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < b_end;
+                                                BrickIt it, int64_t b_begin, int64_t b_end, int64_t zero_to) {
+    const bool zero_rest = zero_to > 0;
+    const int64_t v0 = zero_rest ? 0 : b_begin, v1 = zero_rest ? zero_to : b_end;
+    for (int64_t b = v0 + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < v1;
          b += (int64_t)gridDim.x * blockDim.x) {
         float4* F = reinterpret_cast<float4*>(fb + 8 * b);
         float4* C = reinterpret_cast<float4*>(cb + 8 * b);
+        if (zero_rest && (b < b_begin || b >= b_end)) {
+            C[0] = make_float4(0.f, 0.f, 0.f, 0.f);
+            C[1] = make_float4(0.f, 0.f, 0.f, 0.f);
+            continue;
+        }
         const float4* S = reinterpret_cast<const float4*>(sb + 8 * b);
         float4 f0 = F[0], f1 = F[1];
         const float4 c0 = __ldcs(C), c1 = __ldcs(C + 1), s0 = __ldg(S), s1 = __ldg(S + 1);
