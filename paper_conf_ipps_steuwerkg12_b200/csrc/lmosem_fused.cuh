@@ -10,7 +10,8 @@
 //      not the CTAs of one rank, so no CTA may touch bricks another CTA still reads).
 // Replaces reduce-scatter + update + all-gather; NVLink bytes per GPU with multimem are
 // ~2*|c|/P instead of ~2*(P-1)/P*|c|. Opt-in (LMOSEM_COMBINE_FUSED): with one GPU per test
-// call only the 1-rank peer-pointer path can be exercised here.
+// call only the 1-rank NCCL peer-pointer path can run here; the body (combine_fused_body in
+// lmosem_kernels.cuh) is also run with 2-8 emulated ranks on one GPU (tests/cuda/combine_emu.cu).
 #pragma once
 #include <cuda/atomic>
 #include <nccl.h>
@@ -35,27 +36,20 @@ __device__ __forceinline__ void mm_st4(float* p, float4 v) {
                  : "memory");
 }
 
-__device__ __forceinline__ float4 add4(float4 a, float4 b) { return make_float4(a.x + b.x, a.y + b.y, a.z + b.z, a.w + b.w); }
-
-__device__ __forceinline__ float4 upd4(float4 f, float4 c, float4 s) {
-    return make_float4(upd1(f.x, c.x, s.x), upd1(f.y, c.y, s.y), upd1(f.z, c.z, s.z), upd1(f.w, c.w, s.w));
-}
-
-// One CTA per LSA barrier index. Rank q owns bricks [q*chunk, min((q+1)*chunk, nb)).
+// The NCCL LSA team (one NVLink domain) for combine_fused_body: symmetric windows over c
+// and the brick f; multimem (NVLS, in-switch reduction) when the team has it, else loads
+// and stores to every peer's window.
 template <bool MM>
-__global__ void __launch_bounds__(256) k_combine_fused(ncclDevComm dc, ncclWindow_t wc, ncclWindow_t wf,
-                                                       const float* __restrict__ sb, float* __restrict__ c_local,
-                                                       const float* __restrict__ fb_local, int64_t chunk, int64_t nb) {
-    {
-        ncclLsaBarrierSession<ncclCoopCta> bar(ncclCoopCta(), dc, ncclTeamTagLsa(), blockIdx.x, MM);
+struct NcclTeam {
+    ncclDevComm dc;
+    ncclWindow_t wc, wf;
+    __device__ __forceinline__ void sync(int k) {
+        ncclLsaBarrierSession<ncclCoopCta> bar(ncclCoopCta(), dc, ncclTeamTagLsa(), k, MM);
         bar.sync(ncclCoopCta(), cuda::memory_order_acq_rel);
     }
-    const int nr = dc.lsaSize;
-    const int64_t b0 = chunk * dc.lsaRank, b1 = b0 + chunk < nb ? b0 + chunk : nb;
-    const int64_t t0 = (int64_t)blockIdx.x * blockDim.x + threadIdx.x, stride = (int64_t)gridDim.x * blockDim.x;
-    for (int64_t b = b0 + t0; b < b1; b += stride) {
-        const size_t off = (size_t)b * 32;
-        float4 c0, c1;
+    __device__ __forceinline__ int rank() const { return dc.lsaRank; }
+    __device__ __forceinline__ int size() const { return dc.lsaSize; }
+    __device__ __forceinline__ void sum_c(size_t off, float4& c0, float4& c1) {
         if (MM) {
             const float* pc = (const float*)ncclGetLsaMultimemPointer(wc, off, dc);
             c0 = mm_ld_reduce4(pc);
@@ -63,41 +57,35 @@ __global__ void __launch_bounds__(256) k_combine_fused(ncclDevComm dc, ncclWindo
         } else {
             c0 = make_float4(0.f, 0.f, 0.f, 0.f);
             c1 = c0;
-            for (int p = 0; p < nr; ++p) {
+            for (int p = 0; p < dc.lsaSize; ++p) {
                 const float4* pc = (const float4*)ncclGetLsaPointer(wc, off, p);
                 c0 = add4(c0, pc[0]);
                 c1 = add4(c1, pc[1]);
             }
         }
-        const float4* F = reinterpret_cast<const float4*>(fb_local + 8 * b);
-        const float4* S = reinterpret_cast<const float4*>(sb + 8 * b);
-        const float4 n0 = upd4(F[0], c0, __ldg(S)), n1 = upd4(F[1], c1, __ldg(S + 1));
+    }
+    __device__ __forceinline__ void store_f(size_t off, float4 n0, float4 n1) {
         if (MM) {
             float* pf = (float*)ncclGetLsaMultimemPointer(wf, off, dc);
             mm_st4(pf, n0);
             mm_st4(pf + 4, n1);
         } else {
-            for (int p = 0; p < nr; ++p) {
+            for (int p = 0; p < dc.lsaSize; ++p) {
                 float4* pf = (float4*)ncclGetLsaPointer(wf, off, p);
                 pf[0] = n0;
                 pf[1] = n1;
             }
         }
     }
-    {
-        ncclLsaBarrierSession<ncclCoopCta> bar(ncclCoopCta(), dc, ncclTeamTagLsa(), blockIdx.x, MM);
-        bar.sync(ncclCoopCta(), cuda::memory_order_acq_rel);
-    }
-    // CTA k of every rank has read its bricks of every c: re-zero those bricks locally
-    float4* C = reinterpret_cast<float4*>(c_local);
-    const float4 z = make_float4(0.f, 0.f, 0.f, 0.f);
-    for (int q = 0; q < nr; ++q) {
-        const int64_t q0 = chunk * q, q1 = q0 + chunk < nb ? q0 + chunk : nb;
-        for (int64_t b = q0 + t0; b < q1; b += stride) {
-            C[2 * b] = z;
-            C[2 * b + 1] = z;
-        }
-    }
+};
+
+// One CTA per LSA barrier index.
+template <bool MM>
+__global__ void __launch_bounds__(256) k_combine_fused(ncclDevComm dc, ncclWindow_t wc, ncclWindow_t wf,
+                                                       const float* __restrict__ sb, float* __restrict__ c_local,
+                                                       const float* __restrict__ fb_local, int64_t chunk, int64_t nb) {
+    NcclTeam<MM> team{dc, wc, wf};
+    combine_fused_body(team, blockIdx.x, gridDim.x, sb, c_local, fb_local, chunk, nb);
 }
 
 }  // namespace lmk

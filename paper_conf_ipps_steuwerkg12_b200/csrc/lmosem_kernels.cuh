@@ -619,4 +619,50 @@ __global__ void __launch_bounds__(256) k_update(float* __restrict__ fb, float* _
     }
 }
 
+// ------------------------------------------------------- fused ISD combine (NEXT-1) body
+// The paper's PSD -> ISD switch (Listing 3 l.15-19) as one pass over
+// peer memory, generic over the rank team T (lmosem_fused.cuh: the NCCL LSA team over NVLink;
+// tests/cuda/combine_emu.cu: P emulated ranks on one GPU):
+//   T::sync(k)              barrier of CTA k across the ranks (acquire-release)
+//   T::rank(), T::size()
+//   T::sum_c(off, c0, c1)   the brick at byte offset off of c, summed over the ranks
+//   T::store_f(off, n0, n1) the new brick of f, written to every rank
+// Rank q owns bricks [q*chunk, min((q+1)*chunk, nb)); CTA k of ctas strides over them.
+__device__ __forceinline__ float4 add4(float4 a, float4 b) { return make_float4(a.x + b.x, a.y + b.y, a.z + b.z, a.w + b.w); }
+
+__device__ __forceinline__ float4 upd4(float4 f, float4 c, float4 s) {
+    return make_float4(upd1(f.x, c.x, s.x), upd1(f.y, c.y, s.y), upd1(f.z, c.z, s.z), upd1(f.w, c.w, s.w));
+}
+
+template <class T>
+__device__ __forceinline__ void combine_fused_body(T team, int cta, int ctas, const float* __restrict__ sb,
+                                                   float* __restrict__ c_local, const float* __restrict__ fb_local,
+                                                   int64_t chunk, int64_t nb) {
+    team.sync(cta);  // every rank's projection has finished writing its c
+    const int nr = team.size();
+    const int64_t b0 = chunk * team.rank(), b1 = b0 + chunk < nb ? b0 + chunk : nb;
+    const int64_t t0 = (int64_t)cta * blockDim.x + threadIdx.x, stride = (int64_t)ctas * blockDim.x;
+    for (int64_t b = b0 + t0; b < b1; b += stride) {
+        const size_t off = (size_t)b * 32;
+        float4 c0, c1;
+        team.sum_c(off, c0, c1);
+        const float4* F = reinterpret_cast<const float4*>(fb_local + 8 * b);
+        const float4* S = reinterpret_cast<const float4*>(sb + 8 * b);
+        const float4 n0 = upd4(F[0], c0, __ldg(S)), n1 = upd4(F[1], c1, __ldg(S + 1));
+        team.store_f(off, n0, n1);
+    }
+    team.sync(cta);  // CTA k of every rank has read its bricks of every c and written f
+    // re-zero, in the local c, exactly the bricks CTA k read on every rank (the barrier
+    // orders CTA k across ranks, not the CTAs of one rank)
+    float4* C = reinterpret_cast<float4*>(c_local);
+    const float4 z = make_float4(0.f, 0.f, 0.f, 0.f);
+    for (int q = 0; q < nr; ++q) {
+        const int64_t q0 = chunk * q, q1 = q0 + chunk < nb ? q0 + chunk : nb;
+        for (int64_t b = q0 + t0; b < q1; b += stride) {
+            C[2 * b] = z;
+            C[2 * b + 1] = z;
+        }
+    }
+}
+
 }  // namespace lmk
