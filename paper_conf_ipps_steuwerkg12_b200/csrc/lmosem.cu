@@ -234,11 +234,11 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
         }
     int b = 0;
     switch (mode) {
-        case 0: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<0>, lmk::PROJ_THREADS, smem)); break;
-        case 1: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<1>, lmk::PROJ_THREADS, smem)); break;
-        case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2>, lmk::PROJ_THREADS, smem)); break;
-        case 3: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<3>, lmk::PROJ_THREADS, smem)); break;
-        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<4>, lmk::PROJ_THREADS, smem)); break;
+        case 0: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<0>, lmk::proj_threads_of(0), smem)); break;
+        case 1: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<1>, lmk::proj_threads_of(1), smem)); break;
+        case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2>, lmk::proj_threads_of(2), smem)); break;
+        case 3: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<3>, lmk::proj_threads_of(3), smem)); break;
+        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<4>, lmk::proj_threads_of(4), smem)); break;
     }
     b = std::max(1, b);
     ctx->occ.push_back({mode, smem, b});
@@ -248,11 +248,12 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
 
 lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
     const int cap = launch_cap(mode, g);
-    const size_t sm = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)cap;
+    const int threads = lmk::proj_threads_of(mode);
+    const size_t sm = (threads / 32) * sizeof(int2) * (size_t)cap;
     int per_sm = 1;
     lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm);
     if (s) return s;
-    const int64_t wpb = lmk::PROJ_THREADS / 32;
+    const int64_t wpb = threads / 32;
     const int64_t resident = (int64_t)ctx->num_sms * per_sm * wpb;
     // events per claim: 32 when every warp gets >= 4 claims, else smaller (>= 4); the
     // kernel shrinks its claims further towards the end of the launch (guided)
@@ -265,11 +266,11 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     unsigned long long* work = ctx->work + 2 * ctx->work_next;
     ctx->work_next = (ctx->work_next + 1) % kWorkSlots;
     switch (mode) {
-        case 0: lmk::k_project<0><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        case 1: lmk::k_project<1><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        case 2: lmk::k_project<2><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        case 3: lmk::k_project<3><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        default: lmk::k_project<4><<<grid, lmk::PROJ_THREADS, sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 0: lmk::k_project<0><<<grid, lmk::proj_threads_of(0), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 1: lmk::k_project<1><<<grid, lmk::proj_threads_of(1), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 2: lmk::k_project<2><<<grid, lmk::proj_threads_of(2), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 3: lmk::k_project<3><<<grid, lmk::proj_threads_of(3), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        default: lmk::k_project<4><<<grid, lmk::proj_threads_of(4), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
     }
     CK(cudaGetLastError());
     ctx->st.launches++;

@@ -344,8 +344,11 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #ifndef LMK_GUIDED_DIV
 #define LMK_GUIDED_DIV 2  // guided claims: remaining / (LMK_GUIDED_DIV * warps); 0 = fixed claims
 #endif
+#ifndef LMK_SLAB_CTA_THREADS
+#define LMK_SLAB_CTA_THREADS 128  // CTA size of the z-slab passes (modes 2, 3)
+#endif
 #ifndef LMK_SLAB_MIN_BLOCKS
-#define LMK_SLAB_MIN_BLOCKS LMK_MIN_BLOCKS  // CTAs per SM of the z-slab passes (modes 2, 3)
+#define LMK_SLAB_MIN_BLOCKS 7  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 #ifndef LMK_TRACE
@@ -363,6 +366,11 @@ __device__ __forceinline__ unsigned long long gtimer() {
 #endif
 template <int MODE>
 constexpr int proj_min_blocks() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN_BLOCKS : LMK_MIN_BLOCKS; }
+template <int MODE>
+constexpr int proj_threads() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_CTA_THREADS : LMK_CTA_THREADS; }
+__host__ __device__ constexpr int proj_threads_of(int mode) {
+    return (mode == 2 || mode == 3) ? LMK_SLAB_CTA_THREADS : LMK_CTA_THREADS;
+}
 
 // Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2
 // (<= 3 per dominant-axis slab of the launch's clip box; MODEs 1/2 keep no path: only the
@@ -377,7 +385,7 @@ constexpr int proj_min_blocks() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
 template <int MODE>
-__global__ void __launch_bounds__(PROJ_THREADS, proj_min_blocks<MODE>()) k_project(const float* __restrict__ events, int64_t n,
+__global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>()) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap,
                                                              unsigned long long* __restrict__ work, int batch) {
