@@ -199,6 +199,9 @@ int n_slabs(const lmosem_ctx* ctx) {
 #ifndef LMOSEM_STATIC_BATCH
 #define LMOSEM_STATIC_BATCH 1  // first claim size from the launch's events per warp
 #endif
+#ifndef LMOSEM_FUSED_CTAS_PER_SM
+#define LMOSEM_FUSED_CTAS_PER_SM 4  // fused combine: CTAs (and LSA barriers) per SM
+#endif
 #ifndef LMOSEM_MIN_BATCH
 #define LMOSEM_MIN_BATCH 4
 #endif
@@ -670,7 +673,7 @@ LMOSEM_API lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode) {
             return (ctx->win_c = nullptr, LMOSEM_ENCCL);
         if (!ctx->win_fb && ncclCommWindowRegister(ctx->comm, ctx->fb, bytes, &ctx->win_fb, NCCL_WIN_COLL_SYMMETRIC) != ncclSuccess)
             return (ctx->win_fb = nullptr, LMOSEM_ENCCL);
-        ctx->fused_ctas = ctx->num_sms;
+        ctx->fused_ctas = LMOSEM_FUSED_CTAS_PER_SM * ctx->num_sms;  // all co-resident (barrier per CTA)
         ncclDevCommRequirements reqs;
         std::memset(&reqs, 0, sizeof(reqs));
         reqs.lsaBarrierCount = ctx->fused_ctas;

@@ -64,6 +64,31 @@ struct NcclTeam {
             }
         }
     }
+    __device__ __forceinline__ void sum_c2(size_t oa, size_t ob, float4& a0, float4& a1, float4& b0, float4& b1) {
+        if (MM) {
+            const float* pa = (const float*)ncclGetLsaMultimemPointer(wc, oa, dc);
+            const float* pb = (const float*)ncclGetLsaMultimemPointer(wc, ob, dc);
+            a0 = mm_ld_reduce4(pa);
+            a1 = mm_ld_reduce4(pa + 4);
+            b0 = mm_ld_reduce4(pb);
+            b1 = mm_ld_reduce4(pb + 4);
+        } else {
+            a0 = make_float4(0.f, 0.f, 0.f, 0.f);
+            a1 = a0;
+            b0 = a0;
+            b1 = a0;
+            for (int p = 0; p < dc.lsaSize; ++p) {
+                const char* base = (const char*)ncclGetLsaPointer(wc, 0, p);
+                const float4* pa = (const float4*)(base + oa);
+                const float4* pb = (const float4*)(base + ob);
+                const float4 x0 = pa[0], x1 = pa[1], y0 = pb[0], y1 = pb[1];
+                a0 = add4(a0, x0);
+                a1 = add4(a1, x1);
+                b0 = add4(b0, y0);
+                b1 = add4(b1, y1);
+            }
+        }
+    }
     __device__ __forceinline__ void store_f(size_t off, float4 n0, float4 n1) {
         if (MM) {
             float* pf = (float*)ncclGetLsaMultimemPointer(wf, off, dc);

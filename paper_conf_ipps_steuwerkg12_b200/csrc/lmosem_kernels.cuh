@@ -634,6 +634,7 @@ __global__ void __launch_bounds__(256) k_update(float* __restrict__ fb, float* _
 //   T::sync(k)              barrier of CTA k across the ranks (acquire-release)
 //   T::rank(), T::size()
 //   T::sum_c(off, c0, c1)   the brick at byte offset off of c, summed over the ranks
+//   T::sum_c2(oa, ob, ...)  two bricks at once (loads of both in flight)
 //   T::store_f(off, n0, n1) the new brick of f, written to every rank
 // Rank q owns bricks [q*chunk, min((q+1)*chunk, nb)); CTA k of ctas strides over them.
 __device__ __forceinline__ float4 add4(float4 a, float4 b) { return make_float4(a.x + b.x, a.y + b.y, a.z + b.z, a.w + b.w); }
@@ -650,7 +651,22 @@ __device__ __forceinline__ void combine_fused_body(T team, int cta, int ctas, co
     const int nr = team.size();
     const int64_t b0 = chunk * team.rank(), b1 = b0 + chunk < nb ? b0 + chunk : nb;
     const int64_t t0 = (int64_t)cta * blockDim.x + threadIdx.x, stride = (int64_t)ctas * blockDim.x;
-    for (int64_t b = b0 + t0; b < b1; b += stride) {
+    // two bricks per thread per iteration: their c sums are in flight together
+    int64_t b = b0 + t0;
+    for (; b + stride < b1; b += 2 * stride) {
+        const size_t oa = (size_t)b * 32, ob = (size_t)(b + stride) * 32;
+        float4 ca0, ca1, cb0, cb1;
+        team.sum_c2(oa, ob, ca0, ca1, cb0, cb1);
+        const float4* Fa = reinterpret_cast<const float4*>(fb_local + 8 * b);
+        const float4* Fb = reinterpret_cast<const float4*>(fb_local + 8 * (b + stride));
+        const float4* Sa = reinterpret_cast<const float4*>(sb + 8 * b);
+        const float4* Sb = reinterpret_cast<const float4*>(sb + 8 * (b + stride));
+        const float4 na0 = upd4(Fa[0], ca0, __ldg(Sa)), na1 = upd4(Fa[1], ca1, __ldg(Sa + 1));
+        const float4 nb0 = upd4(Fb[0], cb0, __ldg(Sb)), nb1 = upd4(Fb[1], cb1, __ldg(Sb + 1));
+        team.store_f(oa, na0, na1);
+        team.store_f(ob, nb0, nb1);
+    }
+    if (b < b1) {
         const size_t off = (size_t)b * 32;
         float4 c0, c1;
         team.sum_c(off, c0, c1);

@@ -39,6 +39,10 @@ struct EmuTeam {
             c1 = lmk::add4(c1, __ldcg(pc + 1));
         }
     }
+    __device__ __forceinline__ void sum_c2(size_t oa, size_t ob, float4& a0, float4& a1, float4& b0, float4& b1) {
+        sum_c(oa, a0, a1);
+        sum_c(ob, b0, b1);
+    }
     __device__ __forceinline__ void store_f(size_t off, float4 n0, float4 n1) {
         for (int p = 0; p < P; ++p) {
             float4* pf = reinterpret_cast<float4*>(reinterpret_cast<char*>(f[p]) + off);
@@ -65,7 +69,7 @@ int main() {
     for (int P : {1, 2, 3, 4, 8}) {
         for (int64_t nb : nbs) {
             const int64_t nb_alloc = (nb + P - 1) / P * P, chunk = nb_alloc / P, nbf = 8 * nb_alloc;
-            const int ctas = 148 / P < 1 ? 1 : 148 / P;
+            const int ctas = 4 * 148 / P;  // all P x ctas CTAs co-resident (4 per SM), as in production
             // host images per rank: c (partial error images), brick f (identical replicas), s
             std::vector<std::vector<float>> c(P, std::vector<float>(nbf)), f(P), s(P);
             std::vector<float> f0(nbf), s0(nbf);
