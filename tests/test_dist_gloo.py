@@ -1,4 +1,4 @@
-"""Multi-process (world size 2, gloo, CPU) tests of the N > 1 host logic.
+"""Multi-process (world size 2 and 4, gloo, CPU) tests of the N > 1 host logic.
 
 The GPU path's distribution (§IV.A) is: every rank
 gets the whole subset, projects its block [floor(rN/P), floor((r+1)N/P)) (block
@@ -72,8 +72,8 @@ def _worker(rank, world, port, q):
         dist.destroy_process_group()
 
 
-def test_psd_two_ranks_gloo():
-    world = 2
+@pytest.mark.parametrize("world", [2, 4])
+def test_psd_ranks_gloo(world):
     port = _free_port()
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
@@ -84,8 +84,8 @@ def test_psd_two_ranks_gloo():
     for p in procs:
         p.join(timeout=60)
         assert p.exitcode == 0
-    (r0, b0, e0, same0, err0, *d0), (r1, b1, e1, same1, err1, *d1) = res
-    assert (b0, e0, b1, e1) == (0, 5000, 5000, 10000)
-    assert same0 and same1
-    assert err0 <= 1e-12 and err1 <= 1e-12
-    assert d0[:3] == [0, 2, 128] and d1[:3] == [1, 2, 128] and d0[3] and d1[3]
+    n = 10000
+    for r, (rank, b, e, same, err, d_rank, d_world, id_len, ids_equal) in enumerate(res):
+        assert rank == r and (b, e) == ((r * n) // world, ((r + 1) * n) // world)
+        assert same and err <= 1e-12
+        assert (d_rank, d_world, id_len) == (r, world, 128) and ids_equal
