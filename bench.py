@@ -411,20 +411,27 @@ def main():
     proj_avg_s = proj_ms * 1e-3
     nbf = 8 * ((cfg.dims[0] + 5) // 2) * ((cfg.dims[1] + 5) // 2) * ((cfg.dims[2] + 5) // 2)  # padded bricks
     l2 = l2_peak_gbs(cfg.n_voxels, nbf)
-    alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0  # 4 B gather + 4 B RED per path element, 24 B/event
+    n_slabs = rec.slabs
+    # 4 B gather + 4 B RED per path element, 24 B per event and read (the z-slab form reads
+    # the events in each of its 2 x n_slabs launches)
+    alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)
     traffic, sectors = None, None
     try:
         with open(os.path.join(ROOT, "profiles", "r01_traffic.json")) as fh:
-            t = json.load(fh).get(name)
-        if t:
-            traffic = t["dram_bytes_read_per_launch"] + t["dram_bytes_write_per_launch"]
-            sectors = t["l2_sectors_read_per_launch"] + t["l2_sectors_red_per_launch"]
+            tr = json.load(fh).get(name)
+        if tr and tr.get("launches_per_step", 1) == (2 * n_slabs if n_slabs > 1 else 1):
+            traffic = tr["dram_bytes_read_per_launch"] + tr["dram_bytes_write_per_launch"]
+            sectors = tr["l2_sectors_read_per_launch"] + tr["l2_sectors_red_per_launch"]
     except (OSError, ValueError, KeyError):
         pass
-    roof = {"kernel": "k_project<0> (fused Siddon + forward + back-projection)", "bound": "l2",
+    kname = ("k_project<0> (fused Siddon + forward + back-projection)" if n_slabs == 1 else
+             f"k_project<2>/<3> (z-slab form: {n_slabs} forward-projection + {n_slabs} back-projection launches per "
+             f"subset, summed)")
+    roof = {"kernel": kname, "bound": "l2",
             "achieved": alg_l2_bytes / proj_avg_s / 1e9, "unit": "GB/s", "traffic": traffic,
-            "traffic_note": "DRAM bytes per launch (ncu --set full, profiles/r01_traffic.json); the algorithmic "
-                            "bytes are L2 traffic, the images stay L2-resident",
+            "traffic_note": "DRAM bytes per launch, summed over one subset's launches in the z-slab form (ncu --set "
+                            "full, profiles/r01_traffic.json); the algorithmic bytes are L2 traffic (the images, or "
+                            "the slab being projected, stay L2-resident)",
             "per_unit": f"{mean_path} path elements x (4 B f gather + 4 B c RED) + 24 B event per event",
             "units_per_launch": ev_per_launch}
     if l2:
@@ -436,7 +443,18 @@ def main():
         roof["frac_vs_random_pairs"] = roof["achieved"] / (l2["pair"] * 8.0 / 1e9)
         roof["l2_micro_ops_per_s"] = l2
     roof_sec = None
-    if l2 and sectors:
+    if l2 and sectors and n_slabs > 1:
+        # z-slab form: the gathers (pass A) and the REDs (pass B) run in separate launches,
+        # each bound by its own access type's sector rate -> a two-pass ceiling
+        g_sec, r_sec = tr["l2_sectors_read_per_launch"], tr["l2_sectors_red_per_launch"]
+        t_ceil = g_sec / l2["ldg"] + r_sec / l2["red"]
+        roof_sec = {"bound": "l2_sectors_two_pass", "achieved": sectors / proj_avg_s, "peak": sectors / t_ceil,
+                    "unit": "sectors/s", "frac": t_ceil / proj_avg_s, "sectors_per_launch": sectors,
+                    "path_elements_per_sector": 2 * pairs / sectors,
+                    "what": "ncu L2 sectors of one subset's z-slab launches (gathers in pass A, REDs in pass B) / live "
+                            "projection time, vs the two-pass ceiling gathers / random-gather rate + REDs / random-RED "
+                            "rate (live L2 microbenchmarks)"}
+    elif l2 and sectors:
         # sector view: the L2 moves 32-byte sectors; both microbenchmarks (random and fully
         # coalesced gather+RED pairs) saturate at the same sector rate
         peak_sec = max(l2["red"], l2["ldg"], l2["pair"] * 2.0, l2["pair_run8"] * 2.0 / 8.0,
@@ -447,7 +465,8 @@ def main():
                     "what": "ncu L2 sectors of k_project (gathers + REDs, profiles/r01_traffic.json) / live duration, "
                             "vs the max sector rate over the live L2 microbenchmark modes (random RED, random gather, "
                             "random / 8-lane / 32-lane gather+RED pairs)"}
-    hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0) / proj_avg_s / 1e9, "peak": peaks["hbm_gbs"],
+    hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)) / proj_avg_s / 1e9,
+           "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
     hbm["frac"] = hbm["achieved"] / hbm["peak"]
     # k_update per step: read fb, c, s and write fb, c over the padded brick image (20 B per
