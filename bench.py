@@ -63,7 +63,10 @@ def parse():
     ap.add_argument("--config", default=None, help="C2 (N=1 default), C3 (N>1 default), C4, C5")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
-    ap.add_argument("--cpu-sample", type=int, default=200_000, help="events in the oracle's timed sample")
+    ap.add_argument("--cpu-sample", type=int, default=1_000_000,
+                    help="events in cpu_baseline's timed oracle sample (C2: the whole subset, ~15 s of CPU work)")
+    ap.add_argument("--ref-sample", type=int, default=200_000,
+                    help="events per step of --impl reference (each step a bounded sample of the subset)")
     ap.add_argument("--slabs", type=int, default=0, help="z-slab passes for step 1 (0 = automatic)")
     ap.add_argument("--e2e-file", action="store_true",
                     help="also time lmosem_reconstruct_file from a raw list-mode file (page cache)")
@@ -176,7 +179,7 @@ def cpu_baseline(cfg, sample: int):
     dt = time.perf_counter() - t0
     return {"value": sample / dt, "unit": "events/s", "cores": oracle.get_threads(), "kind": "oracle",
             "sample": f"{sample} events of subset 0 of {cfg.name} (one subset step incl. the {cfg.n_voxels}-voxel "
-                      f"update), {dt:.2f} s wall"}
+                      f"update), {dt:.2f} s wall, {dt * oracle.get_threads():.1f} core-s"}
 
 
 def run_reference(args, cfg, rank):
@@ -184,7 +187,7 @@ def run_reference(args, cfg, rank):
         return
     import oracle
     oracle.set_threads(host_cores())  # rank 0 alone runs: all host cores
-    sample = min(args.cpu_sample, cfg.n_events)
+    sample = min(args.ref_sample, cfg.n_events)
     g = oracle.geom(cfg.dims, cfg.voxel_mm)
     s = lmgen.norm(cfg)
     evs = [lmgen.subset_events(cfg, l % cfg.n_subsets, sample) for l in range(min(cfg.n_subsets, args.warmup + args.steps))]
