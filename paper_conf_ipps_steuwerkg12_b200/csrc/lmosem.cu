@@ -11,6 +11,7 @@
 #include <cerrno>
 #include <cmath>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <new>
 #include <string>
@@ -69,6 +70,14 @@ struct lmosem_ctx {
     bool dev_comm_ok = false, dev_comm_mm = false;
     int fused_ctas = 0;
     int num_sms = 0;
+    // programmatic dependent launch (PDL): a kernel enqueued right after one of ours may
+    // start its independent prologue (claims, event tiles, float64 LOR setup) while its
+    // predecessor drains; it waits (griddepcontrol.wait) before touching f, c or fp.
+    // after_kernel: the last operation this library enqueued on `stream` was one of its own
+    // kernels (reset by every API entry and every non-kernel operation, so a PDL launch
+    // never follows a copy, memset, event, NCCL call or the caller's own work)
+    bool pdl = true;
+    bool after_kernel = false;
     struct Occ {
         int mode;
         size_t smem;
@@ -152,7 +161,31 @@ bool device_accessible(const void* a, const void* b, const void* c = nullptr) {
     do {                                                                                            \
         if (!(ctx)) return LMOSEM_EINVAL;                                                           \
         if ((ctx)->failed) return LMOSEM_ESTATE;                                                    \
+        (ctx)->after_kernel = false;                                                                \
     } while (0)
+
+// Launch one of the library's kernels on ctx->stream, as a programmatic dependent launch
+// when it directly follows another of ours (see lmosem_ctx::pdl).
+template <typename... KArgs, typename... Args>
+cudaError_t launch_k(lmosem_ctx* ctx, void (*kernel)(KArgs...), int grid, int block, size_t smem, Args... args) {
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = 1;
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3((unsigned)grid);
+    cfg.blockDim = dim3((unsigned)block);
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = ctx->stream;
+    cfg.attrs = at;
+    cfg.numAttrs = (ctx->pdl && ctx->after_kernel) ? 1 : 0;
+    const cudaError_t e = cudaLaunchKernelEx(&cfg, kernel, static_cast<KArgs>(args)...);
+    ctx->after_kernel = (e == cudaSuccess);
+    if (e == cudaSuccess) ctx->st.launches++;
+    return e;
+}
+
+// any operation on ctx->stream that is not one of the library's kernels
+inline void not_kernel(lmosem_ctx* ctx) { ctx->after_kernel = false; }
 
 void block_range(int64_t n, int r, int P, int64_t* b, int64_t* e) {
     // floor(r*n/P) without overflow for n < 2^62 / P
@@ -171,16 +204,13 @@ int combine_mode(const lmosem_ctx* ctx) {
 }
 
 lmosem_status launch_to_brick(lmosem_ctx* ctx, const float* row, float* br) {
-    lmk::k_row_to_brick<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(row, br, ctx->geom, ctx->bricks);
-    CK(cudaGetLastError());
-    ctx->st.launches++;
+    CK(launch_k(ctx, lmk::k_row_to_brick, grid_for(ctx, ctx->bricks.nb), 256, 0, row, br, ctx->geom, ctx->bricks));
     return LMOSEM_OK;
 }
 
 lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
-    lmk::k_brick_to_row<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(br, row, ctx->geom, ctx->bricks, zero);
-    CK(cudaGetLastError());
-    ctx->st.launches++;
+    CK(launch_k(ctx, lmk::k_brick_to_row, grid_for(ctx, ctx->bricks.nb), 256, 0, br, row, ctx->geom, ctx->bricks,
+                zero));
     return LMOSEM_OK;
 }
 
@@ -268,15 +298,15 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, max_grid));
     unsigned long long* work = ctx->work + 2 * ctx->work_next;
     ctx->work_next = (ctx->work_next + 1) % kWorkSlots;
+    void (*k)(const float*, int64_t, const float*, float*, float*, lmk::GridGeom, int, unsigned long long*, int);
     switch (mode) {
-        case 0: lmk::k_project<0><<<grid, lmk::proj_threads_of(0), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        case 1: lmk::k_project<1><<<grid, lmk::proj_threads_of(1), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        case 2: lmk::k_project<2><<<grid, lmk::proj_threads_of(2), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        case 3: lmk::k_project<3><<<grid, lmk::proj_threads_of(3), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
-        default: lmk::k_project<4><<<grid, lmk::proj_threads_of(4), sm, ctx->stream>>>(evf, n, ctx->fb, ctx->c, fp, g, cap, work, batch); break;
+        case 0: k = lmk::k_project<0>; break;
+        case 1: k = lmk::k_project<1>; break;
+        case 2: k = lmk::k_project<2>; break;
+        case 3: k = lmk::k_project<3>; break;
+        default: k = lmk::k_project<4>; break;
     }
-    CK(cudaGetLastError());
-    ctx->st.launches++;
+    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch));
     return LMOSEM_OK;
 }
 
@@ -309,6 +339,7 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         CKA(cudaMalloc(&ctx->fp_acc, sizeof(float) * n));
         ctx->fp_cap = n;
     }
+    not_kernel(ctx);
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
     for (int pass = 2; pass <= 3; ++pass)
         for (int k = 0; k < K; ++k)
@@ -323,15 +354,16 @@ lmosem_status launch_update(lmosem_ctx* ctx, float* f_row, int64_t b_begin = 0, 
     if (b_end < 0) b_end = ctx->bricks.nb;
     const int64_t items = zero_to > 0 ? zero_to : b_end - b_begin;
     if (items <= 0) return LMOSEM_OK;
-    lmk::k_update<<<grid_for(ctx, items), 256, 0, ctx->stream>>>(ctx->fb, ctx->c, ctx->norm, f_row, ctx->geom,
-                                                                 ctx->bricks, b_begin, b_end, zero_to);
-    CK(cudaGetLastError());
-    ctx->st.launches++;
+    CK(launch_k(ctx, lmk::k_update, grid_for(ctx, items), 256, 0, ctx->fb, ctx->c, (const float*)ctx->norm, f_row,
+                ctx->geom, ctx->bricks, b_begin, b_end, zero_to));
     return LMOSEM_OK;
 }
 
 lmosem_status mark(lmosem_ctx* ctx, PhaseMarks* pm, int k) {
-    if (pm) CK(cudaEventRecord(pm->e[k], ctx->stream));
+    if (pm) {
+        not_kernel(ctx);
+        CK(cudaEventRecord(pm->e[k], ctx->stream));
+    }
     return LMOSEM_OK;
 }
 
@@ -381,6 +413,7 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         for (int q = 0; q < pipe.in_chunks; ++q) {
             int64_t qb, qe;
             block_range(e - b, q, pipe.in_chunks, &qb, &qe);
+            not_kernel(ctx);
             CK(cudaStreamWaitEvent(ctx->stream, ctx->ev_pipe[q], 0));
             if ((s = launch_project(ctx, ev + b + qb, qe - qb, nullptr, 0))) return s;
         }
@@ -392,6 +425,7 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         // NEXT-1: reduce-scatter + update + all-gather as one kernel over peer memory
         const int64_t chunk = ctx->nb_alloc / ctx->world;
         if ((s = mark(ctx, pm, 3))) return s;
+        not_kernel(ctx);  // launched plainly: its LSA barriers order it across the ranks
         if (ctx->dev_comm_mm)
             lmk::k_combine_fused<true><<<ctx->fused_ctas, 256, 0, ctx->stream>>>(
                 ctx->dev_comm, ctx->win_c, ctx->win_fb, ctx->norm, ctx->c, ctx->fb, chunk, ctx->bricks.nb);
@@ -406,15 +440,19 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         // holds the sum over its brick block, update only that block, all-gather f.
         const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
         float* my_c = ctx->c + 8 * b0;
+        not_kernel(ctx);
         NK(ncclReduceScatter(ctx->c, my_c, (size_t)(8 * chunk), ncclFloat32, ncclSum, ctx->comm, ctx->stream));
         if ((s = mark(ctx, pm, 3))) return s;
         // one launch: the block update (re-zeroes its c) and c <- 0 on every other brick
         if ((s = launch_update(ctx, nullptr, b0, std::min(b0 + chunk, ctx->bricks.nb), ctx->nb_alloc))) return s;
+        not_kernel(ctx);
         NK(ncclAllGather(ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk), ncclFloat32, ctx->comm, ctx->stream));
         if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
     } else {
-        if (ctx->comm)
+        if (ctx->comm) {
+            not_kernel(ctx);
             NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+        }
         if ((s = mark(ctx, pm, 3))) return s;
         if (write_f && pipe.host_f) {
             // z-ranges of bricks: bricks [z0, z1) * BX*BY hold rows iz in [2 z0 - 2, 2 z1 - 2)
@@ -427,6 +465,7 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
                 const int64_t r0 = std::max<int64_t>(0, 2 * z0 - lmk::HALO_LO);
                 const int64_t r1 = std::min<int64_t>(ctx->dims[2], 2 * z1 - lmk::HALO_LO);
                 if (r1 <= r0) continue;
+                not_kernel(ctx);
                 CK(cudaEventRecord(ctx->ev_pipe[q], ctx->stream));
                 CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_pipe[q], 0));
                 CK(cudaMemcpyAsync(pipe.host_f + r0 * rowp, f + r0 * rowp, sizeof(float) * (size_t)((r1 - r0) * rowp),
@@ -586,6 +625,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cudaDeviceProp prop;
     if (!cuda(cudaGetDeviceProperties(&prop, ctx->device), "cudaGetDeviceProperties")) return bail(s);
     ctx->num_sms = prop.multiProcessorCount;
+    if (const char* e = std::getenv("LMOSEM_PDL")) ctx->pdl = e[0] != '0';  // A/B switch (default on)
     if (ctx->proj_smem > (size_t)prop.sharedMemPerBlockOptin) {
         ctx->err = "volume too large for the shared-memory path buffer";
         return bail(LMOSEM_EINVAL);
@@ -857,6 +897,7 @@ LMOSEM_API lmosem_status lmosem_reconstruct_file(lmosem_ctx* ctx, const char* pa
                 s = fail(ctx, LMOSEM_EIO, std::string("reconstruct_file: read ") + path + ": " + strerror(errno));
                 break;
             }
+            not_kernel(ctx);  // the wait on ctx->stream below
             if (cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_consumed[k], 0) != cudaSuccess ||
                 (e > b && cudaMemcpyAsync(ctx->dev_ev[k], ctx->pin_ev[k], sizeof(lmosem_event) * (e - b),
                                           cudaMemcpyHostToDevice, ctx->copy_stream) != cudaSuccess) ||
@@ -902,6 +943,7 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
             const int k = (int)(step & 1);
             int64_t b, e;
             block_range(offsets[l + 1] - offsets[l], ctx->rank, ctx->world, &b, &e);
+            not_kernel(ctx);  // the event record / wait on ctx->stream around this subset
             CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_consumed[k], 0));
             cudaEvent_t h0 = nullptr, h1 = nullptr;
             if (ctx->timing) {
@@ -983,7 +1025,10 @@ LMOSEM_API lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event*
     block_range(n_events, ctx->rank, ctx->world, &b, &e);
     lmosem_status s;
     if ((s = launch_project(ctx, events + b, e - b, nullptr, 4))) return s;
-    if (ctx->comm) NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    if (ctx->comm) {
+        not_kernel(ctx);
+        NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+    }
     return launch_to_row(ctx, ctx->c, s_out, 1);  // s_out <- c, c <- 0
 }
 

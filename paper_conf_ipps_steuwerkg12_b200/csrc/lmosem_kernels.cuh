@@ -364,6 +364,15 @@ __device__ __forceinline__ unsigned long long gtimer() {
     return t;
 }
 #endif
+// Programmatic dependent launch (the host launches a kernel that directly follows another
+// of the library's with programmaticStreamSerialization; without it both are no-ops):
+// pdl_trigger lets the next kernel in the stream start launching its CTAs (they occupy
+// an SM only as this kernel's CTAs leave it); pdl_wait blocks until every prerequisite
+// grid has completed and its memory is visible. Each kernel waits before its first
+// access to an image or per-event array that an earlier kernel writes or reads.
+__device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+
 template <int MODE>
 constexpr int proj_min_blocks() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN_BLOCKS : LMK_MIN_BLOCKS; }
 template <int MODE>
@@ -404,6 +413,11 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     // left a tail of that length at the end of every launch
     const int64_t warps_in_grid = (int64_t)gridDim.x * (blockDim.x >> 5);
     int take = batch;
+    pdl_trigger();
+    // claims, event tiles and the float64 setup of the first LORs overlap the previous
+    // kernel's tail; pass B reads fp during setup, so it waits at once
+    bool dep_ready = MODE == 3;
+    if (MODE == 3) pdl_wait();
 #if LMK_TRACE
     const int gw = blockIdx.x * (blockDim.x >> 5) + wib;
     unsigned long long tr_start = gtimer(), tr_first = 0, tr_lors = 0, tr_claims = 0;
@@ -465,6 +479,10 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 fp_known = fp[idx];
                 ok = ok && fp_known > 0.0f;  // reading S7
             }
+        }
+        if (!dep_ready) {  // warp-uniform
+            pdl_wait();
+            dep_ready = true;
         }
         if (MODE == 1 && mine_ev && !ok) fp[idx] = 0.0f;
         __syncwarp();  // the tile is dead: the path buffer may be overwritten
@@ -540,6 +558,8 @@ __device__ __forceinline__ bool real_voxel(const GridGeom& g, int px, int py, in
 // row (x-fastest, caller) -> bricks (halo = 0)
 __global__ void __launch_bounds__(256) k_row_to_brick(const float* __restrict__ row, float* __restrict__ br,
                                                       GridGeom g, BrickIt it) {
+    pdl_wait();
+    pdl_trigger();
     for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
         const int bx = (int)(b % it.BX);
         const int64_t t = b / it.BX;
@@ -559,6 +579,8 @@ __global__ void __launch_bounds__(256) k_row_to_brick(const float* __restrict__ 
 // bricks -> row (real voxels only); optionally zeroes the bricks afterwards
 __global__ void __launch_bounds__(256) k_brick_to_row(float* __restrict__ br, float* __restrict__ row, GridGeom g,
                                                       BrickIt it, int zero) {
+    pdl_wait();
+    pdl_trigger();
     for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
         const int bx = (int)(b % it.BX);
         const int64_t t = b / it.BX;
@@ -591,6 +613,8 @@ __device__ __forceinline__ float upd1(float f, float c, float s) {
 __global__ void __launch_bounds__(256) k_update(float* __restrict__ fb, float* __restrict__ cb,
                                                 const float* __restrict__ sb, float* __restrict__ f_row, GridGeom g,
                                                 BrickIt it, int64_t b_begin, int64_t b_end, int64_t zero_to) {
+    pdl_wait();
+    pdl_trigger();
     const bool zero_rest = zero_to > 0;
     const int64_t v0 = zero_rest ? 0 : b_begin, v1 = zero_rest ? zero_to : b_end;
     for (int64_t b = v0 + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < v1;
