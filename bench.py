@@ -413,8 +413,11 @@ def main():
     pairs = ev_per_launch * mean_path
     proj_avg_s = proj_ms * 1e-3
     nbf = 8 * ((cfg.dims[0] + 5) // 2) * ((cfg.dims[1] + 5) // 2) * ((cfg.dims[2] + 5) // 2)  # padded bricks
-    l2 = l2_peak_gbs(cfg.n_voxels, nbf)
     n_slabs = rec.slabs
+    # the microbenchmarks run on a buffer of the size each projection launch works on: the
+    # image (V floats), or in the z-slab form one slab of the brick image (L2-resident)
+    l2_floats = cfg.n_voxels if n_slabs == 1 else nbf // n_slabs
+    l2 = l2_peak_gbs(l2_floats, nbf)
     # 4 B gather + 4 B RED per path element, 24 B per event and read (the z-slab form reads
     # the events in each of its 2 x n_slabs launches)
     alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)
@@ -440,8 +443,8 @@ def main():
     if l2:
         roof["peak"] = l2["pair_warp32"] * 8.0 / 1e9
         roof["peak_kind"] = ("measured live: fully coalesced fp32 gather+RED pairs (each warp on 32 consecutive "
-                             "floats) on a V-float L2-resident buffer (libl2peak.so, PAIR_WARP32); the random-"
-                             "address pair rate is l2_micro_ops_per_s.pair")
+                             f"floats) on a {l2_floats}-float L2-resident buffer (the image, or one z-slab of it; libl2peak.so, "
+                             "PAIR_WARP32); the random-address pair rate is l2_micro_ops_per_s.pair")
         roof["frac"] = roof["achieved"] / roof["peak"]
         roof["frac_vs_random_pairs"] = roof["achieved"] / (l2["pair"] * 8.0 / 1e9)
         roof["l2_micro_ops_per_s"] = l2

@@ -727,3 +727,31 @@ def test_runtime_failure_poisons_context():
     st1, st2, st3 = (int(x) for x in lines[0].split()[:3])
     assert st1 == 0 and st2 == 3 and st3 == 5, lines
     assert lines[-1] == "destroy 0"
+
+
+@pytest.mark.parametrize("slabs", [1, 3])
+def test_programmatic_dependent_launch_on_off(pkg, monkeypatch, slabs):
+    """The kernels of a reconstruction run as programmatic dependent launches (each waits,
+    griddepcontrol.wait, before touching f, c or fp); LMOSEM_PDL=0 (read at lmosem_init)
+    launches them plainly. Both orders reach the oracle's 3-subset result, and agree."""
+    cfg = lmgen.CONFIGS["C2"]
+    L, n = 3, 200_000
+    ev = np.concatenate([lmgen.subset_events(cfg, l, n) for l in range(L)])
+    s = lmgen.norm(cfg)
+    off = np.arange(L + 1) * n
+    f0 = np.random.default_rng(5).uniform(0.5, 2.0, cfg.n_voxels).astype(np.float32)
+    got = {}
+    for pdl in ("0", "1"):
+        monkeypatch.setenv("LMOSEM_PDL", pdl)
+        rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+        rec.set_slabs(slabs)
+        f = dev(f0)
+        rec.reconstruct(dev(ev), off, 1, f)
+        rec.synchronize()
+        got[pdl] = f.cpu().numpy().astype(np.float64)
+        rec.close()
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, f0.astype(np.float64))
+    for pdl in ("0", "1"):
+        assert maxrel(got[pdl], ref) <= 2 * MAXREL_SUBSET
+        assert rel_l2(got[pdl], ref) <= REL_L2_RECON
+    assert maxrel(got["1"], got["0"]) <= 1e-5
