@@ -351,6 +351,9 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #define LMK_SLAB_MIN_BLOCKS 7  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
+#ifndef LMK_SETUP_ONLY
+#define LMK_SETUP_ONLY 0  // diagnostic builds only: skip the traversal (setup cost)
+#endif
 #ifndef LMK_TRACE
 #define LMK_TRACE 0  // diagnostic builds only (tools/trace_tail.py): per-warp timeline
 #endif
@@ -487,6 +490,17 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         if (MODE == 1 && mine_ev && !ok) fp[idx] = 0.0f;
         __syncwarp();  // the tile is dead: the path buffer may be overwritten
         unsigned mask = __ballot_sync(0xffffffffu, ok);
+#if LMK_SETUP_ONLY
+        // diagnostic builds only (tools/ab_variants.py setup_only): claims, tiles and the
+        // float64 setup without the traversal (the result is kept live, never stored)
+        if (ok) {
+            const unsigned h = (unsigned)mine.wb0 ^ (unsigned)mine.wc0 ^ (unsigned)mine.sb ^ (unsigned)mine.sc ^
+                               __float_as_uint(mine.ab + mine.ac + mine.lunit + mine.fin + mine.fout) ^
+                               (unsigned)(mine.i0 ^ mine.ns ^ mine.code);
+            if (h == 0x9e3779b9u) cb[0] += 1.0f;
+        }
+        mask = 0;
+#endif
 #if LMK_TRACE
         tr_claims++;
         if (!tr_first && mask) tr_first = gtimer();
