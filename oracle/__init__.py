@@ -49,7 +49,9 @@ _P = ctypes.c_void_p
 def _load():
     global _lib
     if _lib is None:
-        lib = ctypes.CDLL(build())
+        # LMOSEM_ORACLE_SO: a prebuilt variant of this library (tests/test_oracle_mutants.py
+        # loads deliberately broken copies to check that the pins catch them)
+        lib = ctypes.CDLL(os.environ.get("LMOSEM_ORACLE_SO") or build())
         G = ctypes.POINTER(Geom)
         for name in ("oracle_siddon_path", "oracle_boxclip_path"):
             fn = getattr(lib, name)

@@ -78,6 +78,12 @@ def test_golden_paths(case):
     coord, ln = oracle.siddon_path(G4, p1, p2)
     assert coord.tolist() == [c for c, _ in pairs]
     np.testing.assert_allclose(ln, [l for _, l in pairs], rtol=1e-13, atol=1e-14)
+    # the brute-force box clip (the reference routine of P2/P10/P14) reaches the same
+    # hand-derived path, face cases included (half-open voxel boxes, reading S6)
+    bc, bl = oracle.boxclip_path(G4, p1, p2)
+    got = dict(zip(bc.tolist(), bl.tolist()))
+    assert sorted(got) == sorted(c for c, _ in pairs)
+    np.testing.assert_allclose([got[c] for c, _ in pairs], [l for _, l in pairs], rtol=1e-13, atol=1e-14)
 
 
 def test_golden_em_update():
@@ -297,6 +303,41 @@ def test_p10_sparse_matrix_em():
     exp = np.where((c > 0) & (s > 0), f0 * c / np.where(s > 0, s, 1), f0)
     got = oracle.subset_step(g, ev, s, f0)
     np.testing.assert_allclose(got, exp, rtol=1e-12)
+
+
+# ---------------------------------------------------------------- P15 ordered subsets
+def test_p15_ordered_subsets_em():
+    """OSEM (Listing 2 line 1: the subsets in order, each an EM update from the
+    previous one's image; lines 591-593: the pass over the subsets repeated): three unequal
+    subsets x two iterations, each step the Shepp-Vardi update with that subset's A from the
+    brute-force clip via scipy.sparse, vs oracle.reconstruct with the subsets' offsets."""
+    sp = pytest.importorskip("scipy.sparse")
+    dims, vox = (5, 6, 4), (1.1, 0.9, 1.0)
+    g = oracle.geom(dims, vox)
+    V = int(np.prod(dims))
+    rng = np.random.default_rng(15)
+    lors = random_lors(rng, dims, vox, 90)
+    ev = np.array([np.concatenate([a, b]) for a, b in lors], np.float32)
+    offsets = np.array([0, 20, 55, 90], np.int64)
+    s = rng.uniform(0.3, 1.2, V).astype(np.float32)
+    f0 = rng.uniform(0.5, 1.5, V)
+    A_of = []
+    for l in range(3):
+        rows, cols, vals = [], [], []
+        for r, i in enumerate(range(offsets[l], offsets[l + 1])):
+            co, ln = oracle.boxclip_path(g, ev[i, :3], ev[i, 3:])
+            rows += [r] * len(co)
+            cols += co.tolist()
+            vals += ln.tolist()
+        A_of.append(sp.csr_matrix((vals, (rows, cols)), shape=(offsets[l + 1] - offsets[l], V)))
+    exp = f0.copy()
+    for _ in range(2):
+        for A in A_of:
+            Af = A @ exp
+            c = A.T @ np.where(Af > 0, 1.0 / np.where(Af > 0, Af, 1), 0.0)
+            exp = np.where((c > 0) & (s > 0), exp * c / s, exp)
+    got = oracle.reconstruct(g, ev, offsets, 2, s, f0)
+    np.testing.assert_allclose(got, exp, rtol=1e-11)
 
 
 # ---------------------------------------------------------------- P11 EM monotonicity
