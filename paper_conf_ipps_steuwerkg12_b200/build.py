@@ -51,9 +51,12 @@ def build_l2peak() -> str:
     return L2PEAK_SO
 
 
-def build(force: bool = False, verbose: bool = False, defines=(), out: str | None = None) -> str:
+def build(force: bool = False, verbose: bool = False, defines=(), out: str | None = None,
+          csrc: str | None = None) -> str:
     """Builds liblmosem.so (and libl2peak.so). `defines`/`out` build an A/B variant of
-    the kernels (e.g. defines=["LMK_TRASH=0"], out=".../liblmosem_v.so")."""
+    the kernels (e.g. defines=["LMK_TRASH=0"], out=".../liblmosem_v.so"); `csrc` compiles
+    a modified copy of the sources (tools/gpu_mutants.py) into `out`."""
+    src_dir = csrc or CSRC
     if out is None and not force and not needs_build():
         return SO
     target = out or SO
@@ -63,8 +66,8 @@ def build(force: bool = False, verbose: bool = False, defines=(), out: str | Non
     tmp = target + f".tmp{os.getpid()}"
     cmd = [NVCC, *ARCH, "-O3", "-std=c++17", "-lineinfo", "-Xptxas", "-v", *[f"-D{d}" for d in defines],
            "-Xcompiler", "-fPIC,-fvisibility=hidden", "-shared",
-           "-I", os.path.join(ROOT, "include"), "-I", CSRC, "-I", inc,
-           os.path.join(CSRC, "lmosem.cu"), "-o", tmp,
+           "-I", os.path.join(ROOT, "include"), "-I", src_dir, "-I", inc,
+           os.path.join(src_dir, "lmosem.cu"), "-o", tmp,
            "-L", lib, "-l:libnccl.so.2", f"-Xlinker=-rpath={lib}", "-lpthread"]
     res = subprocess.run(cmd, capture_output=True, text=True)
     if res.returncode != 0:

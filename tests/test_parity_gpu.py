@@ -615,7 +615,7 @@ def test_pathological_coordinates_do_not_fault(pkg):
     rec.close()
 
 
-@pytest.mark.parametrize("vox", [(0.3, 0.7, 1.1), (0.45, 1.3, 0.9), (1.0, 1.0, 1.0)])
+@pytest.mark.parametrize("vox", [(0.3, 0.7, 1.1), (0.45, 1.3, 0.9), (1.0, 1.0, 1.0), (0.3, 0.9, 1.1)])
 def test_lors_in_voxel_faces(pkg, vox):
     """Axis-parallel LORs lying exactly in voxel faces (float32 coordinates nearest to the
     planes lo + k*v, as crystal grids produce): the voxel row is a floating-point decision,
@@ -630,8 +630,11 @@ def test_lors_in_voxel_faces(pkg, vox):
         a = i % 3
         b, c = (a + 1) % 3, (a + 2) % 3
         p = np.zeros(3)
-        p[b] = lo[b] + rng.integers(0, dims[b] + 1) * vox[b]  # a face (or the outer faces)
-        p[c] = lo[c] + rng.integers(0, dims[c] + 1) * vox[c] if i % 2 else rng.uniform(lo[c], -lo[c])
+        # every face plane of axis b in turn (or the outer faces); (0.3, 0.9, 1.1): with 16
+        # voxels of 0.9 mm the face k = 13 is one where floor((p - lo) * (1/v)) would be
+        # one row lower than floor((p - lo) / v)
+        p[b] = lo[b] + ((i // 3) % (dims[b] + 1)) * vox[b]
+        p[c] = lo[c] + ((i // 7) % (dims[c] + 1)) * vox[c] if i % 2 else rng.uniform(lo[c], -lo[c])
         q = p.copy()
         p[a], q[a] = lo[a] - 3.0, -lo[a] + 3.0
         ev.append(np.concatenate([p, q]))
@@ -755,3 +758,31 @@ def test_programmatic_dependent_launch_on_off(pkg, monkeypatch, slabs):
         assert maxrel(got[pdl], ref) <= 2 * MAXREL_SUBSET
         assert rel_l2(got[pdl], ref) <= REL_L2_RECON
     assert maxrel(got["1"], got["0"]) <= 1e-5
+
+
+@pytest.mark.parametrize("slabs", [1, 3])
+def test_zero_forward_projection_events_skipped(pkg, slabs):
+    """Reading S7 (the division at PAPER.md line 464): an event whose forward projection is
+    0 (its path only crosses voxels with f = 0) contributes nothing. f0 is zero outside a
+    small ball, so most C1 events have fp = 0; the fused kernel and the z-slab passes must
+    skip them (otherwise c = inf and f = 0 * inf = NaN on their paths)."""
+    cfg, ev, s = inputs("C1")
+    ev = ev[:cfg.n_events]
+    nx, ny, nz = cfg.dims
+    i = np.arange(cfg.n_voxels)
+    ix, iy, iz = i % nx, (i // nx) % ny, i // (nx * ny)
+    f0 = np.where((ix - 9) ** 2 + (iy - 7) ** 2 + (iz - 8) ** 2 <= 4, 1.5, 0.0).astype(np.float32)
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    fp = oracle.forward(g, ev, f0)
+    assert (fp == 0).sum() > len(ev) // 2 and (fp > 0).sum() > 50  # both kinds present
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    rec.set_slabs(slabs)
+    f = dev(f0)
+    rec.subset_step(dev(ev), f)
+    rec.synchronize()
+    rec.close()
+    got = f.cpu().numpy().astype(np.float64)
+    ref = oracle.subset_step(g, ev, s, f0)
+    assert np.all(np.isfinite(got))
+    assert np.array_equal(got == 0, ref == 0)
+    assert maxrel(got, ref) <= MAXREL_SUBSET
