@@ -351,6 +351,10 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #define LMK_SLAB_MIN_BLOCKS 7  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
+#ifndef LMK_GEOM_UNROLL
+#define LMK_GEOM_UNROLL 0  // unroll of the geometry loop (0 = the compiler's choice, 2x)
+#endif
+constexpr int kGeomUnroll = LMK_GEOM_UNROLL > 0 ? LMK_GEOM_UNROLL : 1;
 #ifndef LMK_SETUP_ONLY
 #define LMK_SETUP_ONLY 0  // diagnostic builds only: skip the traversal (setup cost)
 #endif
@@ -517,6 +521,9 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             int cnt = 0;
             float acc = 0.0f;
             Step S = make_step(L, W, lane);
+#if LMK_GEOM_UNROLL > 0
+#pragma unroll (kGeomUnroll)
+#endif
             for (int k0 = 0; k0 < L.ns; k0 += 32, advance(S)) {
                 const int k = k0 + lane;
                 const bool in = k < L.ns;  // lanes past the last slab compute garbage, store nothing

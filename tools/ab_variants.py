@@ -12,7 +12,10 @@ VARIANTS = {
     # compile-time switches left in the kernel: LMK_CTA_THREADS, LMK_MIN_BLOCKS
     # (rejected variants are listed with their numbers in DESIGN.md §7)
     "default": [],
-    "setup_only": ["LMK_SETUP_ONLY=1"],  # diagnostic: claims + tiles + float64 setup, no traversal
+    "setup_only": ["LMK_SETUP_ONLY=1"],
+    "unroll1": ["LMK_GEOM_UNROLL=1"],
+    "unroll3": ["LMK_GEOM_UNROLL=3"],
+    "unroll4": ["LMK_GEOM_UNROLL=4"],  # diagnostic: claims + tiles + float64 setup, no traversal
     "c256x2": ["LMK_MIN_BLOCKS=2"],
     "slab4": ["LMK_SLAB_MIN_BLOCKS=4"],
     "guided1": ["LMK_GUIDED_DIV=1"],
