@@ -471,6 +471,20 @@ def main():
                     "what": "ncu L2 sectors of k_project (gathers + REDs, profiles/r01_traffic.json) / live duration, "
                             "vs the max sector rate over the live L2 microbenchmark modes (random RED, random gather, "
                             "random / 8-lane / 32-lane gather+RED pairs)"}
+    # request view (DESIGN.md §7 summary): the SM->L2 request interface takes about one request
+    # cycle per SM clock; a gather request (any sectors of one 128-byte line) costs one cycle,
+    # a RED one cycle per 32-byte sector (tools/request_probe.cu)
+    roof_req = None
+    clocks = clk.summary()
+    if n_slabs == 1 and sectors and tr.get("l2_requests_read_per_launch"):
+        sm_hz = (clocks.get("sm_mhz") or peaks.get("sm_max_mhz") or 1965.0) * 1e6
+        cyc = tr["l2_requests_read_per_launch"] + tr["l2_sectors_red_per_launch"]
+        peak_req = torch.cuda.get_device_properties(dev).multi_processor_count * sm_hz
+        roof_req = {"bound": "l2_request_interface", "achieved": cyc / proj_avg_s, "peak": peak_req,
+                    "unit": "request cycles/s", "frac": cyc / proj_avg_s / peak_req,
+                    "request_cycles_per_launch": cyc, "ncu_req_cycles_active_pct": tr.get("req_cycles_active_pct"),
+                    "what": "(gather requests + RED sectors) per launch (ncu, profiles/r01_traffic.json) / live "
+                            "duration, vs one request cycle per SM clock (SMs x median SM clock under load)"}
     hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)) / proj_avg_s / 1e9,
            "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
@@ -508,9 +522,10 @@ def main():
                               "steps": K2, "ms_per_step_instrumented": instr_ms,
                               "what": "library CUDA events around each phase on its stream, in an instrumented pass "
                                       "of the same loop right after the timed region"},
-        "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_hbm_events": hbm, "roofline_update": upd,
+        "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_l2_requests": roof_req,
+        "roofline_hbm_events": hbm, "roofline_update": upd,
         "gpu_launches": launches, "flushed_subset_step": flushed, "per_rank_share": shares,
-        "clocks": clk.summary(), "wall_s_timed_region": t_wall,
+        "clocks": clocks, "wall_s_timed_region": t_wall,
         "e2e": e2e,
         "paper_context": PAPER_CONTEXT,
     }

@@ -44,6 +44,10 @@ def main(rep, summary, config="C2", per_step=1):
         "source": f"profiles/{summary}",
         "l2_sectors_read_per_launch": tot("lts__t_sectors_srcunit_tex_op_read.sum"),
         "l2_sectors_red_per_launch": tot("lts__t_sectors_srcunit_tex_op_red.sum"),
+        "l2_requests_read_per_launch": tot("lts__t_requests_srcunit_tex_op_read.sum"),
+        "l2_requests_red_per_launch": tot("lts__t_requests_srcunit_tex_op_red.sum"),
+        "req_cycles_active_pct": round(sum(num(r, "l1tex__m_l1tex2xbar_req_cycles_active.avg.pct_of_peak_sustained_elapsed")
+                                           for r in rows) / len(rows), 2),
     }
     try:
         with open(PATH) as fh:
