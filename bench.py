@@ -166,6 +166,17 @@ def host_cores() -> int:
         return os.cpu_count() or 1
 
 
+def cpu_model() -> str:
+    try:
+        with open("/proc/cpuinfo") as fh:
+            for ln in fh:
+                if ln.startswith("model name"):
+                    return ln.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
 def cpu_baseline(cfg, sample: int):
     """The float64 oracle as it stands, on this host's cores, on a bounded sample."""
     import oracle
@@ -178,6 +189,7 @@ def cpu_baseline(cfg, sample: int):
     oracle.subset_step(g, ev, s, f0)
     dt = time.perf_counter() - t0
     return {"value": sample / dt, "unit": "events/s", "cores": oracle.get_threads(), "kind": "oracle",
+            "cpu_model": cpu_model(), "nproc": os.cpu_count(),
             "sample": f"{sample} events of subset 0 of {cfg.name} (one subset step incl. the {cfg.n_voxels}-voxel "
                       f"update), {dt:.2f} s wall, {dt * oracle.get_threads():.1f} core-s"}
 
@@ -207,6 +219,7 @@ def run_reference(args, cfg, rank):
                                             f"{cfg.dims[2]}, subsets of {cfg.n_events} events (oracle steps use a "
                                             f"{sample}-event sample of each subset)"},
             "cpu_baseline": {"value": v, "unit": "events/s", "cores": cores, "kind": "oracle",
+                             "cpu_model": cpu_model(), "nproc": os.cpu_count(),
                              "sample": f"{sample} events per step x {args.steps} steps"},
             "e2e": {"value": v, "unit": "events/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
