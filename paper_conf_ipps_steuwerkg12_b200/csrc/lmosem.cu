@@ -34,9 +34,13 @@ struct PhaseMarks {
 
 }  // namespace
 
-// reconstruct_host pipelines the first subset's event upload and the final f download
-// in kPipe chunks (hides ~0.8 ms per C2 reconstruction)
+// reconstruct_host pipelines the final f download in kPipe brick z-ranges
 constexpr int kPipe = 8;
+// the first subset's upload: kInChunks parts of growing size (1/16, 3/16, 4/16, 8/16 of the
+// events). Pinned H2D (~2.3e9 events/s) outruns the projection (~1e9 events/s), so only the
+// first, small part's upload is exposed, and few launches keep their ramp/tail cost low.
+constexpr int kInChunks = 4;
+constexpr int kInChunkEnd[kInChunks + 1] = {0, 1, 4, 8, 16};  // sixteenths of the events
 
 struct lmosem_ctx {
     int device = -1;
@@ -191,6 +195,17 @@ void block_range(int64_t n, int r, int P, int64_t* b, int64_t* e) {
     // floor(r*n/P) without overflow for n < 2^62 / P
     *b = (int64_t)((__int128)n * r / P);
     *e = (int64_t)((__int128)n * (r + 1) / P);
+}
+
+// part q of Q (1: the whole range; kInChunks: the first subset's growing parts) of n events
+void in_chunk_range(int64_t n, int q, int Q, int64_t* b, int64_t* e) {
+    if (Q == 1) {
+        *b = 0;
+        *e = n;
+        return;
+    }
+    *b = n * kInChunkEnd[q] / 16;
+    *e = n * kInChunkEnd[q + 1] / 16;
 }
 
 int grid_for(lmosem_ctx* ctx, int64_t items) {
@@ -412,7 +427,7 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
     if (pipe.in_chunks > 1) {
         for (int q = 0; q < pipe.in_chunks; ++q) {
             int64_t qb, qe;
-            block_range(e - b, q, pipe.in_chunks, &qb, &qe);
+            in_chunk_range(e - b, q, pipe.in_chunks, &qb, &qe);
             not_kernel(ctx);
             CK(cudaStreamWaitEvent(ctx->stream, ctx->ev_pipe[q], 0));
             if ((s = launch_project(ctx, ev + b + qb, qe - qb, nullptr, 0))) return s;
@@ -960,10 +975,10 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
             }
             HostPipe pipe;
             // nothing to overlap the first subset's upload with: chunk it (>= 64 K events per chunk)
-            if (step == 0 && e - b >= (int64_t)kPipe * 65536) pipe.in_chunks = kPipe;
+            if (step == 0 && e - b >= (int64_t)16 * 16384) pipe.in_chunks = kInChunks;
             for (int q = 0; q < pipe.in_chunks; ++q) {
                 int64_t qb, qe;
-                block_range(e - b, q, pipe.in_chunks, &qb, &qe);
+                in_chunk_range(e - b, q, pipe.in_chunks, &qb, &qe);
                 if (qe > qb)
                     CK(cudaMemcpyAsync(ctx->dev_ev[k] + qb, events + offsets[l] + b + qb, sizeof(lmosem_event) * (qe - qb),
                                        cudaMemcpyHostToDevice, ctx->copy_stream));
