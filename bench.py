@@ -489,15 +489,16 @@ def main():
     # a RED one cycle per 32-byte sector (tools/request_probe.cu)
     roof_req = None
     clocks = clk.summary()
-    if n_slabs == 1 and sectors and tr.get("l2_requests_read_per_launch"):
+    if sectors and tr.get("l2_requests_read_per_launch"):
         sm_hz = (clocks.get("sm_mhz") or peaks.get("sm_max_mhz") or 1965.0) * 1e6
         cyc = tr["l2_requests_read_per_launch"] + tr["l2_sectors_red_per_launch"]
         peak_req = torch.cuda.get_device_properties(dev).multi_processor_count * sm_hz
         roof_req = {"bound": "l2_request_interface", "achieved": cyc / proj_avg_s, "peak": peak_req,
                     "unit": "request cycles/s", "frac": cyc / proj_avg_s / peak_req,
                     "request_cycles_per_launch": cyc, "ncu_req_cycles_active_pct": tr.get("req_cycles_active_pct"),
-                    "what": "(gather requests + RED sectors) per launch (ncu, profiles/r01_traffic.json) / live "
-                            "duration, vs one request cycle per SM clock (SMs x median SM clock under load)"}
+                    "what": "(gather requests + RED sectors) per launch (ncu, profiles/r01_traffic.json; summed over "
+                            "a subset's launches in the z-slab form) / live duration, vs one request cycle per SM "
+                            "clock (SMs x median SM clock under load)"}
     hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)) / proj_avg_s / 1e9,
            "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
