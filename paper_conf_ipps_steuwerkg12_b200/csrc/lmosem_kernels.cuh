@@ -50,6 +50,9 @@ __device__ __forceinline__ int bidx(int A, int B, int p) { return A * p + B * (p
 // stepping w(k) = w0 + k*s, floor = w >> 40, fraction = low 40 bits. The slope error
 // (<= 2^-41 per slab) accumulates to < 1e-9 voxel over 600 slabs.
 constexpr int FIX_BITS = 40;
+#ifndef LMK_SCALE_PIECES
+#define LMK_SCALE_PIECES 0  // 1: scale every piece length to mm in the geometry loop (A/B)
+#endif
 
 // Per-LOR traversal state (broadcast lane -> warp by shuffles; 16 registers).
 struct Lor {
@@ -218,8 +221,8 @@ __device__ __forceinline__ Walk make_walk(const Lor& L, const GridGeom& g) {
     return W;
 }
 
-// The (up to) three pieces of slab k: j = brick index, l = chord length in mm (0 for
-// an empty piece).
+// The (up to) three pieces of slab k: j = brick index, l = chord length in units of the
+// slab along the dominant axis (x lunit = mm; 0 for an empty piece).
 struct Pieces {
     int j0, j1, j2;
     float l0, l1, l2;
@@ -263,9 +266,17 @@ __device__ __forceinline__ Pieces slab_pieces(const Lor& L, const Walk& W, int k
     P.j0 = Ja + Jb0 + Jc0;
     P.j1 = Ja + ((db <= dc) ? (Jb1 + Jc0) : (Jb0 + Jc1));
     P.j2 = Ja + Jb1 + Jc1;
+#if LMK_SCALE_PIECES
     P.l0 = (q1 - dlo) * L.lunit;
     P.l1 = (q2 - q1) * L.lunit;
     P.l2 = (dhi - q2) * L.lunit;
+#else
+    // lengths in units of the slab (u_a); the LOR's mm per unit, lunit, is applied once per
+    // LOR to fp and to the back-projected weight (three multiplies fewer per slab)
+    P.l0 = q1 - dlo;
+    P.l1 = q2 - q1;
+    P.l2 = dhi - q2;
+#endif
     return P;
 }
 
@@ -538,7 +549,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             }
             float fpv = fp_known;
             if (kGather) {
-                fpv = warp_sum(acc);
+                fpv = warp_sum(acc) * (LMK_SCALE_PIECES ? 1.0f : L.lunit);
                 if (MODE == 1 && lane == 0) fp[base + src] = fpv;
                 if (MODE == 2 && lane == 0) fp[base + src] += fpv;
             } else {
@@ -548,7 +559,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             if (kScatter && fpv > 0.0f) {  // reading S7: skip events with fp <= 0
                 // pass 2: back-projection, lane m <- piece m (path order: consecutive
                 // lanes share 32-byte brick sectors)
-                const float inv = 1.0f / fpv;
+                const float inv = (LMK_SCALE_PIECES ? 1.0f : L.lunit) / fpv;
 #pragma unroll 8
                 for (int m = lane; m < cnt; m += 32) {
                     const int2 q = lds2(path_s + 8u * (unsigned)m);
