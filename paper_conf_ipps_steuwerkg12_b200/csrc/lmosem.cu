@@ -286,7 +286,8 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
         case 1: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<1>, lmk::proj_threads_of(1), smem)); break;
         case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2>, lmk::proj_threads_of(2), smem)); break;
         case 3: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<3>, lmk::proj_threads_of(3), smem)); break;
-        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<4>, lmk::proj_threads_of(4), smem)); break;
+        case 4: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<4>, lmk::proj_threads_of(4), smem)); break;
+        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<5>, lmk::proj_threads_of(5), smem)); break;
     }
     b = std::max(1, b);
     ctx->occ.push_back({mode, smem, b});
@@ -319,7 +320,8 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
         case 1: k = lmk::k_project<1>; break;
         case 2: k = lmk::k_project<2>; break;
         case 3: k = lmk::k_project<3>; break;
-        default: k = lmk::k_project<4>; break;
+        case 4: k = lmk::k_project<4>; break;
+        default: k = lmk::k_project<5>; break;
     }
     CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch));
     return LMOSEM_OK;
@@ -340,7 +342,8 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
     if (n <= 0) return LMOSEM_OK;
     const float* evf = reinterpret_cast<const float*>(ev);
     const int K = n_slabs(ctx);
-    if (mode == 1 || K == 1) return launch_mode(ctx, mode, evf, n, fp_out, ctx->geom);
+    if (mode == 1 || K == 1)  // the fused pass gathers through the texture pipe when it can (MODE 5)
+        return launch_mode(ctx, (mode == 0 && ctx->geom.tex_fb) ? 5 : mode, evf, n, fp_out, ctx->geom);
     lmosem_status s;
     if (mode == 4) {
         for (int k = 0; k < K; ++k)
@@ -657,6 +660,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         cuda(cudaFuncSetAttribute(lmk::k_project<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
         cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
         cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<5>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
     }
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
@@ -703,6 +707,27 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     cuda(cudaMemsetAsync(ctx->fb, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset fb");
     cuda(cudaMemsetAsync(ctx->norm, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset norm");
     cuda(cudaMemsetAsync(ctx->work, 0, sizeof(unsigned long long) * 2 * kWorkSlots, ctx->stream), "memset work");
+    // MODE 5 (the fused pass with texture gathers) when the brick f fits a 1-D linear
+    // texture; else, or with LMOSEM_TEX=0 (A/B, tests), the LSU gathers of MODE 0
+    const char* te = std::getenv("LMOSEM_TEX");
+    int max_lin = 0;
+    cudaDeviceGetAttribute(&max_lin, cudaDevAttrMaxTexture1DLinearWidth, ctx->device);
+    if (s == LMOSEM_OK && !(te && te[0] == '0') && 8 * ctx->nb_alloc <= (int64_t)max_lin) {
+        cudaResourceDesc rd;
+        std::memset(&rd, 0, sizeof(rd));
+        rd.resType = cudaResourceTypeLinear;
+        rd.res.linear.devPtr = ctx->fb;
+        rd.res.linear.desc = cudaCreateChannelDesc<float>();
+        rd.res.linear.sizeInBytes = sizeof(float) * 8 * ctx->nb_alloc;
+        cudaTextureDesc td;
+        std::memset(&td, 0, sizeof(td));
+        td.readMode = cudaReadModeElementType;
+        cudaTextureObject_t t = 0;
+        if (cudaCreateTextureObject(&t, &rd, &td, nullptr) == cudaSuccess)
+            ctx->geom.tex_fb = t;
+        else
+            (void)cudaGetLastError();  // not fatal: MODE 0 gathers
+    }
     if (s == LMOSEM_OK) {
         lmk::k_row_to_brick<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->scratch, ctx->norm,
                                                                                      ctx->geom, ctx->bricks);
@@ -1135,6 +1160,7 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     for (auto e : ctx->ev_pipe)
         if (e) cudaEventDestroy(e);
     if (ctx->dev_f) cudaFree(ctx->dev_f);
+    if (ctx->geom.tex_fb) cudaDestroyTextureObject(ctx->geom.tex_fb);
     if (ctx->c) cudaFree(ctx->c);
     if (ctx->fb) cudaFree(ctx->fb);
     if (ctx->norm) cudaFree(ctx->norm);

@@ -41,6 +41,7 @@ struct GridGeom {
     double lo[3];     // volume lower corner (mm): -n*v/2
     double v[3];      // voxel size (mm)
     double inv_v[3];  // 1 / voxel size (1/mm)
+    unsigned long long tex_fb;  // 1-D texture object over the brick f (MODE 5), 0 = none
 };
 
 // J_axis(p) = M*(p>>1) + m*(p&1) = (M/2)*p + (m - M/2)*(p&1), (M, m) = (8,1), (8BX,2), (8BX*BY,4)
@@ -409,6 +410,8 @@ __host__ __device__ constexpr int proj_threads_of(int mode) {
 //         fp[i] from pass A (events with fp <= 0 skipped).
 // MODE 4: sensitivity image: back-projection of ones, cb_j += a_ij (no forward
 //         projection).
+// MODE 5: MODE 0 with the gathers of f through the texture pipe (tex1Dfetch on g.tex_fb),
+//         the default for the fused pass when the brick f fits a 1-D linear texture.
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
 template <int MODE>
@@ -416,8 +419,9 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap,
                                                              unsigned long long* __restrict__ work, int batch) {
-    constexpr bool kGather = MODE <= 2;    // forward projection in this launch
-    constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4;  // back-projection in this launch
+    constexpr bool kGather = MODE <= 2 || MODE == 5;  // forward projection in this launch
+    constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4 || MODE == 5;  // back-projection
+    constexpr bool kTex = MODE == 5;  // gathers of f through the texture path
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
@@ -542,9 +546,17 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
                 if (kScatter) append3(path_s, cnt, lt, P, v0, v1, v2);
                 if (kGather) {
-                    acc = fmaf(v0 ? __ldg(fb + P.j0) : 0.f, P.l0, acc);
-                    acc = fmaf(v1 ? __ldg(fb + P.j1) : 0.f, P.l1, acc);
-                    acc = fmaf(v2 ? __ldg(fb + P.j2) : 0.f, P.l2, acc);
+                    if (kTex) {
+                        // texel index through the texture pipe: the gathers leave the LSU data
+                        // pipe to the REDs and the path buffer
+                        acc = fmaf(v0 ? tex1Dfetch<float>(g.tex_fb, P.j0) : 0.f, P.l0, acc);
+                        acc = fmaf(v1 ? tex1Dfetch<float>(g.tex_fb, P.j1) : 0.f, P.l1, acc);
+                        acc = fmaf(v2 ? tex1Dfetch<float>(g.tex_fb, P.j2) : 0.f, P.l2, acc);
+                    } else {
+                        acc = fmaf(v0 ? __ldg(fb + P.j0) : 0.f, P.l0, acc);
+                        acc = fmaf(v1 ? __ldg(fb + P.j1) : 0.f, P.l1, acc);
+                        acc = fmaf(v2 ? __ldg(fb + P.j2) : 0.f, P.l2, acc);
+                    }
                 }
             }
             float fpv = fp_known;

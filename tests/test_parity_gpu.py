@@ -786,3 +786,26 @@ def test_zero_forward_projection_events_skipped(pkg, slabs):
     assert np.all(np.isfinite(got))
     assert np.array_equal(got == 0, ref == 0)
     assert maxrel(got, ref) <= MAXREL_SUBSET
+
+
+@pytest.mark.parametrize("tex", ["0", "1"])
+def test_lsu_and_texture_gathers(pkg, monkeypatch, tex):
+    """The fused pass gathers f through the texture pipe (MODE 5) when the brick f fits a
+    1-D linear texture, else (or with LMOSEM_TEX=0, read at lmosem_init) with LSU loads
+    (MODE 0): both against the oracle on a C2-sized subset and through a reconstruction."""
+    cfg = lmgen.CONFIGS["C2"]
+    L, n = 2, 200_000
+    ev = np.concatenate([lmgen.subset_events(cfg, l, n) for l in range(L)])
+    s = lmgen.norm(cfg)
+    off = np.arange(L + 1) * n
+    f0 = np.random.default_rng(9).uniform(0.5, 2.0, cfg.n_voxels).astype(np.float32)
+    monkeypatch.setenv("LMOSEM_TEX", tex)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f = dev(f0)
+    rec.reconstruct(dev(ev), off, 1, f)
+    rec.synchronize()
+    rec.close()
+    got = f.cpu().numpy().astype(np.float64)
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, f0.astype(np.float64))
+    assert maxrel(got, ref) <= 2 * MAXREL_SUBSET
+    assert rel_l2(got, ref) <= REL_L2_RECON
