@@ -24,7 +24,15 @@ MUTANTS = [
     ("first-slab clip ignored", K, "const float dlo = (k == 0) ? L.fin : 0.0f;", "const float dlo = 0.0f;", False),
     ("last-slab clip ignored", K, "const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;", "const float dhi = 1.0f;",
      False),
-    ("piece length without mm per slab", K, "P.l0 = (q1 - dlo) * L.lunit;", "P.l0 = (q1 - dlo);", False),
+    ("fp without mm per slab unit", K, "fpv = warp_sum(acc) * (LMK_SCALE_PIECES ? 1.0f : L.lunit);",
+     "fpv = warp_sum(acc);", False),
+    ("back-projected weight without mm per slab unit", K,
+     "const float inv = (LMK_SCALE_PIECES ? 1.0f : L.lunit) / fpv;", "const float inv = 1.0f / fpv;", False),
+    ("texture gather of piece 0 reads piece 1's voxel", K,
+     "acc = fmaf(v0 ? tex1Dfetch<float>(g.tex_fb, P.j0) : 0.f, P.l0, acc);",
+     "acc = fmaf(v0 ? tex1Dfetch<float>(g.tex_fb, P.j1) : 0.f, P.l0, acc);", False),
+    ("LSU gather of piece 2 dropped (MODE 0 / z-slab pass A)", K,
+     "acc = fmaf(v2 ? __ldg(fb + P.j2) : 0.f, P.l2, acc);", "acc = acc;", False),
     ("RED without 1/fp", K, "atomicAdd(cb + q.x, __int_as_float(q.y) * inv);", "atomicAdd(cb + q.x, __int_as_float(q.y));",
      False),
     ("fp <= 0 events not skipped", K, "if (kScatter && fpv > 0.0f) {", "if (kScatter) {", False),
@@ -63,7 +71,7 @@ MUTANTS = [
 # the same events (measured: the mutant passes every parity test, as expected).
 TESTS = ("golden or degenerate or axis_parallel or c1_ or zslab_passes_match_oracle_c1 or odd_extents or "
          "lors_in_voxel_faces or one_subset_paper_shaped or programmatic or nccl_combine_single_rank or "
-         "combine_modes_single_rank or zero_forward_projection")
+         "combine_modes_single_rank or zero_forward_projection or lsu_and_texture")
 
 
 def build():
