@@ -103,6 +103,16 @@ const char* lmosem_version(void);
  * needed. EINVAL if n < 0, world < 1, rank outside [0, world) or a pointer is NULL. */
 lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end);
 
+/* The ISD combine's brick blocks (the PSD -> ISD switch): the
+ * internal image of n_bricks 8-float bricks is allocated as *alloc = n_bricks rounded up to a
+ * multiple of world and split into world equal chunks; rank owns chunk `rank` (its part of
+ * the reduce-scatter, the step-2 update and the all-gather), of which [*begin, *end) are real
+ * bricks (*end <= n_bricks; a trailing chunk may be shorter or empty). Pure host function;
+ * the blocks of ranks 0..world-1 partition [0, n_bricks). EINVAL on null pointers,
+ * n_bricks < 0, world < 1 or rank outside [0, world). */
+lmosem_status lmosem_isd_block(int64_t n_bricks, int32_t rank, int32_t world, int64_t* begin, int64_t* end,
+                               int64_t* alloc);
+
 /* Writes a fresh NCCL unique id (LMOSEM_NCCL_ID_BYTES bytes) to out. ENCCL on failure. */
 lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
 

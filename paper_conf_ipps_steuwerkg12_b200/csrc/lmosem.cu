@@ -208,6 +208,17 @@ void in_chunk_range(int64_t n, int q, int Q, int64_t* b, int64_t* e) {
     *e = n * kInChunkEnd[q + 1] / 16;
 }
 
+// ISD combine blocks: the nb bricks are allocated as `alloc` =
+// nb rounded up to a multiple of world, split into world equal chunks; rank r owns (reduces,
+// updates, all-gathers) chunk r, of which [begin, end) are real bricks (end <= nb)
+void isd_block(int64_t nb, int rank, int world, int64_t* begin, int64_t* end, int64_t* alloc) {
+    const int64_t a = (nb + world - 1) / world * world;
+    const int64_t chunk = a / world;
+    *alloc = a;
+    *begin = std::min(nb, chunk * rank);
+    *end = std::min(nb, chunk * (rank + 1));
+}
+
 int grid_for(lmosem_ctx* ctx, int64_t items) {
     const int64_t cap = (int64_t)ctx->num_sms * 16;
     return (int)std::max<int64_t>(1, std::min<int64_t>((items + 255) / 256, cap));
@@ -457,12 +468,14 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         // PAPER.md lines 509-518 (Listing 3 l.15-19): PSD -> ISD. Reduce-scatter c so rank r
         // holds the sum over its brick block, update only that block, all-gather f.
         const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
+        int64_t blk_b, blk_e, alloc;
+        isd_block(ctx->bricks.nb, ctx->rank, ctx->world, &blk_b, &blk_e, &alloc);
         float* my_c = ctx->c + 8 * b0;
         not_kernel(ctx);
         NK(ncclReduceScatter(ctx->c, my_c, (size_t)(8 * chunk), ncclFloat32, ncclSum, ctx->comm, ctx->stream));
         if ((s = mark(ctx, pm, 3))) return s;
         // one launch: the block update (re-zeroes its c) and c <- 0 on every other brick
-        if ((s = launch_update(ctx, nullptr, b0, std::min(b0 + chunk, ctx->bricks.nb), ctx->nb_alloc))) return s;
+        if ((s = launch_update(ctx, nullptr, blk_b, blk_e, alloc))) return s;
         not_kernel(ctx);
         NK(ncclAllGather(ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk), ncclFloat32, ctx->comm, ctx->stream));
         if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
@@ -555,6 +568,13 @@ LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t wor
     return LMOSEM_OK;
 }
 
+LMOSEM_API lmosem_status lmosem_isd_block(int64_t n_bricks, int32_t rank, int32_t world, int64_t* begin,
+                                          int64_t* end, int64_t* alloc) {
+    if (!begin || !end || !alloc || n_bricks < 0 || world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
+    isd_block(n_bricks, rank, world, begin, end, alloc);
+    return LMOSEM_OK;
+}
+
 LMOSEM_API lmosem_status lmosem_nccl_unique_id(void* out, size_t size) {
     if (!out || size < sizeof(ncclUniqueId) || sizeof(ncclUniqueId) != LMOSEM_NCCL_ID_BYTES) return LMOSEM_EINVAL;
     ncclUniqueId id;
@@ -614,7 +634,10 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     ctx->bricks.BZ = ctx->geom.P[2] / 2;
     ctx->bricks.nb = (int64_t)ctx->bricks.BX * ctx->bricks.BY * ctx->bricks.BZ;
     ctx->nbf = 8 * ctx->bricks.nb;
-    ctx->nb_alloc = (ctx->bricks.nb + world - 1) / world * world;  // equal ISD brick blocks
+    {
+        int64_t b0, b1;
+        isd_block(ctx->bricks.nb, rank, world, &b0, &b1, &ctx->nb_alloc);  // equal ISD brick blocks
+    }
     if (ctx->nbf >= (int64_t(1) << 31)) {
         delete ctx;
         return LMOSEM_EINVAL;

@@ -27,7 +27,7 @@ EXPORTS = (
     "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
     "lmosem_destroy", "lmosem_last_error", "lmosem_set_slabs", "lmosem_get_slabs",
     "lmosem_sensitivity", "lmosem_set_norm", "lmosem_set_combine", "lmosem_get_combine",
-    "lmosem_reconstruct_file",
+    "lmosem_reconstruct_file", "lmosem_isd_block",
 )
 COMBINE_ALLREDUCE, COMBINE_ISD, COMBINE_FUSED = 1, 2, 3
 
@@ -72,6 +72,7 @@ def load(build_if_missing: bool = False) -> ctypes.CDLL:
     sig = {
         "lmosem_version": ([], ctypes.c_char_p),
         "lmosem_block_range": ([_I64, _I32, _I32, ctypes.POINTER(_I64), ctypes.POINTER(_I64)], _S),
+        "lmosem_isd_block": ([_I64, _I32, _I32, ctypes.POINTER(_I64), ctypes.POINTER(_I64), ctypes.POINTER(_I64)], _S),
         "lmosem_nccl_unique_id": ([_P, ctypes.c_size_t], _S),
         "lmosem_init": ([ctypes.POINTER(_P), _P, _P, _P, ctypes.POINTER(Dist)], _S),
         "lmosem_set_stream": ([_P, _P], _S),
@@ -113,6 +114,16 @@ def block_range(n: int, rank: int, world: int) -> tuple[int, int]:
     if st != OK:
         raise LmosemError(st, "block_range: bad arguments")
     return b.value, e.value
+
+
+def isd_block(n_bricks: int, rank: int, world: int) -> tuple[int, int, int]:
+    """(begin, end, alloc) of rank's ISD brick block."""
+    b, e, a = _I64(), _I64(), _I64()
+    st = load().lmosem_isd_block(int(n_bricks), int(rank), int(world), ctypes.byref(b), ctypes.byref(e),
+                                 ctypes.byref(a))
+    if st != OK:
+        raise LmosemError(st, "isd_block: bad arguments")
+    return b.value, e.value, a.value
 
 
 def nccl_unique_id() -> bytes:

@@ -53,6 +53,27 @@ def test_block_range_partition(lib):
     assert pkg.block_range(big, 7, 8) == ((7 * big) // 8, big)
 
 
+def test_isd_block_partition(lib):
+    """The ISD combine's brick blocks (the NCCL reduce-scatter / all-gather chunks and the
+    block update at P > 1): equal chunks of the padded allocation, rank order, real-brick
+    parts partitioning [0, n_bricks)."""
+    import paper_conf_ipps_steuwerkg12_b200 as pkg
+    for nb in (0, 1, 7, 8, 1000, 27 * 10**5 + 13, 6735344):
+        for P in (1, 2, 3, 4, 7, 8):
+            blocks = [pkg.isd_block(nb, r, P) for r in range(P)]
+            alloc = blocks[0][2]
+            assert all(b[2] == alloc for b in blocks)
+            assert alloc % P == 0 and nb <= alloc < nb + P
+            chunk = alloc // P
+            for r, (b, e, _) in enumerate(blocks):
+                assert b == min(nb, r * chunk) and e == min(nb, (r + 1) * chunk)
+            assert blocks[0][0] == 0 and blocks[-1][1] == nb
+            assert all(blocks[r][1] == blocks[r + 1][0] for r in range(P - 1))
+    for bad in ((-1, 0, 1), (10, 1, 1), (10, -1, 2), (10, 0, 0)):
+        with pytest.raises(pkg.LmosemError):
+            pkg.isd_block(*bad)
+
+
 @pytest.mark.parametrize("args", [(-1, 0, 1), (10, -1, 2), (10, 2, 2), (10, 0, 0)])
 def test_block_range_einval(lib, args):
     with pytest.raises(pkg.LmosemError) as e:
