@@ -188,8 +188,10 @@ def cpu_baseline(cfg, sample: int):
     t0 = time.perf_counter()
     oracle.subset_step(g, ev, s, f0)
     dt = time.perf_counter() - t0
+    s_subset = dt * cfg.n_events / sample  # one whole subset at this rate
     return {"value": sample / dt, "unit": "events/s", "cores": oracle.get_threads(), "kind": "oracle",
             "cpu_model": cpu_model(), "nproc": os.cpu_count(),
+            "s_per_subset": s_subset, "s_per_recon": s_subset * cfg.n_subsets,
             "sample": f"{sample} events of subset 0 of {cfg.name} (one subset step incl. the {cfg.n_voxels}-voxel "
                       f"update), {dt:.2f} s wall, {dt * oracle.get_threads():.1f} core-s"}
 
