@@ -51,6 +51,9 @@ __device__ __forceinline__ int bidx(int A, int B, int p) { return A * p + B * (p
 // stepping w(k) = w0 + k*s, floor = w >> 40, fraction = low 40 bits. The slope error
 // (<= 2^-41 per slab) accumulates to < 1e-9 voxel over 600 slabs.
 constexpr int FIX_BITS = 40;
+#ifndef LMK_APPEND2
+#define LMK_APPEND2 0  // 1: path-buffer prefix from two ballots on n = v0 + v1 + v2 (A/B)
+#endif
 #ifndef LMK_SCALE_PIECES
 #define LMK_SCALE_PIECES 0  // 1: scale every piece length to mm in the geometry loop (A/B)
 #endif
@@ -337,14 +340,22 @@ __device__ __forceinline__ int2 lds2(unsigned addr) {
 // path_s: 32-bit shared-window address of the warp's path buffer (8 B per piece).
 __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, const Pieces& P, bool v0, bool v1,
                                         bool v2) {
+#if LMK_APPEND2
+    // exclusive prefix over lanes of n = v0 + v1 + v2 (0..3) from two ballots on its bits
+    const unsigned n = (unsigned)v0 + (unsigned)v1 + (unsigned)v2;
+    const unsigned b0 = __ballot_sync(0xffffffffu, n & 1u), b1 = __ballot_sync(0xffffffffu, n & 2u);
+    const unsigned a = path_s + 8u * (unsigned)(cnt + __popc(b0 & lt) + 2 * __popc(b1 & lt));
+    cnt += __popc(b0) + 2 * __popc(b1);
+#else
     // exclusive prefix over lanes of v0 + v1 + v2 from three predicate ballots
     const unsigned b0 = __ballot_sync(0xffffffffu, v0), b1 = __ballot_sync(0xffffffffu, v1),
                    b2 = __ballot_sync(0xffffffffu, v2);
     const unsigned a = path_s + 8u * (unsigned)(cnt + __popc(b0 & lt) + __popc(b1 & lt) + __popc(b2 & lt));
+    cnt += __popc(b0) + __popc(b1) + __popc(b2);
+#endif
     if (v0) sts2(a, P.j0, P.l0);
     if (v1) sts2(a + (v0 ? 8u : 0u), P.j1, P.l1);
     if (v2) sts2(a + (v0 ? 8u : 0u) + (v1 ? 8u : 0u), P.j2, P.l2);
-    cnt += __popc(b0) + __popc(b1) + __popc(b2);
 }
 
 #ifndef LMK_CTA_THREADS
