@@ -261,6 +261,15 @@ int n_slabs(const lmosem_ctx* ctx) {
 #ifndef LMOSEM_MIN_BATCH
 #define LMOSEM_MIN_BATCH 4
 #endif
+#ifndef LMOSEM_GUIDED_LARGE
+#define LMOSEM_GUIDED_LARGE 3  // guided divisor for launches of >= LMOSEM_GUIDED_ROUNDS rounds of claims
+#endif
+#ifndef LMOSEM_GUIDED_SMALL
+#define LMOSEM_GUIDED_SMALL 2  // ... and for smaller ones (a rank's share at P >= 2); 0 = fixed claims
+#endif
+#ifndef LMOSEM_GUIDED_ROUNDS
+#define LMOSEM_GUIDED_ROUNDS 6  // rounds = events / (32 x resident warps)
+#endif
 #ifndef LMOSEM_CLAIMS
 #define LMOSEM_CLAIMS 4  // target claims per warp
 #endif
@@ -325,7 +334,10 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     const int grid = (int)std::max<int64_t>(1, std::min(blocks_needed, max_grid));
     unsigned long long* work = ctx->work + 2 * ctx->work_next;
     ctx->work_next = (ctx->work_next + 1) % kWorkSlots;
-    void (*k)(const float*, int64_t, const float*, float*, float*, lmk::GridGeom, int, unsigned long long*, int);
+    // guided claims: a full C2/C5 subset (~9 rounds of 32-event claims per warp)
+    // gains from the smaller final claims of divisor 3; a rank's share at P >= 2 from 2
+    const int gdiv = n >= (int64_t)LMOSEM_GUIDED_ROUNDS * 32 * resident ? LMOSEM_GUIDED_LARGE : LMOSEM_GUIDED_SMALL;
+    void (*k)(const float*, int64_t, const float*, float*, float*, lmk::GridGeom, int, unsigned long long*, int, int);
     switch (mode) {
         case 0: k = lmk::k_project<0>; break;
         case 1: k = lmk::k_project<1>; break;
@@ -334,7 +346,7 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
         case 4: k = lmk::k_project<4>; break;
         default: k = lmk::k_project<5>; break;
     }
-    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch));
+    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch, gdiv));
     return LMOSEM_OK;
 }
 

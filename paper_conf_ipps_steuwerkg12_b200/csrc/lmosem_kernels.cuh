@@ -364,9 +364,6 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
-#ifndef LMK_GUIDED_DIV
-#define LMK_GUIDED_DIV 2  // guided claims: remaining / (LMK_GUIDED_DIV * warps); 0 = fixed claims
-#endif
 #ifndef LMK_SLAB_CTA_THREADS
 #define LMK_SLAB_CTA_THREADS 128  // CTA size of the z-slab passes (modes 2, 3)
 #endif
@@ -429,7 +426,8 @@ template <int MODE>
 __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>()) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap,
-                                                             unsigned long long* __restrict__ work, int batch) {
+                                                             unsigned long long* __restrict__ work, int batch,
+                                                             int gdiv) {
     constexpr bool kGather = MODE <= 2 || MODE == 5;  // forward projection in this launch
     constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4 || MODE == 5;  // back-projection
     constexpr bool kTex = MODE == 5;  // gathers of f through the texture path
@@ -441,7 +439,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     // dynamic work distribution: each warp claims consecutive events from a global counter
     // (work[0]; zero at launch), so unequal LOR lengths and small per-rank subsets do not
     // leave idle warps. Guided claim sizes: `batch` (<= 32) while there is plenty of work,
-    // then remaining / (LMK_GUIDED_DIV * warps in the grid), even and >= 2 (claims stay
+    // then remaining / (gdiv * warps in the grid), even and >= 2 (claims stay
     // 16-byte aligned) — a 32-event claim takes a warp ~0.1 ms at C2, so fixed claims
     // left a tail of that length at the end of every launch
     const int64_t warps_in_grid = (int64_t)gridDim.x * (blockDim.x >> 5);
@@ -480,13 +478,11 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         // coalesced 16-byte vector loads into the head of the warp's path buffer (idle at
         // this point), then each lane reads its record from shared memory
         const int m = (int)min((int64_t)take, n - base);
-#if LMK_GUIDED_DIV > 0
-        {
+        if (gdiv > 0) {  // 0: fixed claims
             const int64_t rem = n - base - take;  // work left after this claim (estimate)
-            const int64_t g = rem / (LMK_GUIDED_DIV * warps_in_grid);
+            const int64_t g = rem / (gdiv * warps_in_grid);
             take = batch <= 2 ? batch : (int)max((int64_t)2, min((int64_t)batch, g)) & ~1;
         }
-#endif
         const float* tile_g = events + 6 * base;
         const bool vec = ((((uintptr_t)tile_g) & 15) == 0) && ((m & 1) == 0);
         float4* tile_s = reinterpret_cast<float4*>(smem_path + (size_t)wib * cap);

@@ -20,9 +20,11 @@ VARIANTS = {
     "unroll4": ["LMK_GEOM_UNROLL=4"],  # diagnostic: claims + tiles + float64 setup, no traversal
     "c256x2": ["LMK_MIN_BLOCKS=2"],
     "slab4": ["LMK_SLAB_MIN_BLOCKS=4"],
-    "guided1": ["LMK_GUIDED_DIV=1"],
-    "guided4": ["LMK_GUIDED_DIV=4"],
-    "fixed": ["LMK_GUIDED_DIV=0"],
+    "guided1": ["LMOSEM_GUIDED_LARGE=1", "LMOSEM_GUIDED_SMALL=1"],
+    "guided2": ["LMOSEM_GUIDED_LARGE=2", "LMOSEM_GUIDED_SMALL=2"],
+    "guided3": ["LMOSEM_GUIDED_LARGE=3", "LMOSEM_GUIDED_SMALL=3"],
+    "guided4": ["LMOSEM_GUIDED_LARGE=4", "LMOSEM_GUIDED_SMALL=4"],
+    "fixed": ["LMOSEM_GUIDED_LARGE=0", "LMOSEM_GUIDED_SMALL=0"],
     "nostatic": ["LMOSEM_STATIC_BATCH=0"],
     "min2": ["LMOSEM_MIN_BATCH=2"],
     "claims8": ["LMOSEM_CLAIMS=8", "LMOSEM_MIN_BATCH=2"],
