@@ -90,8 +90,12 @@ typedef struct {
     int64_t timed_subsets; /* subsets covered by the phase times below */
     double convert_ms;     /* f -> internal brick layout (subset_step; first subset of reconstruct) */
     double project_ms;     /* step 1: fused traversal + forward + back-projection kernel */
-    double combine_ms;     /* c all-reduce (world > 1) */
-    double update_ms;      /* step 2: update kernel (also re-zeroes c) */
+    double combine_ms;     /* the combine (world > 1): ALLREDUCE the all-reduce of c; ISD the
+                              reduce-scatter, the block update and the all-gather of f; FUSED
+                              the fused kernel (which includes the block update) */
+    double update_ms;      /* what follows the combine: ALLREDUCE (and one GPU) the step-2 update
+                              kernel (also re-zeroes c); ISD / FUSED the brick -> caller-layout
+                              copy of f (written on the last subset of a reconstruct) */
     double h2d_ms;         /* event uploads in lmosem_reconstruct_host (copy stream) */
 } lmosem_stats;
 
@@ -143,9 +147,31 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  * peer loads), updates it and writes the new f block to every rank (multimem.st or peer
  * stores), between two LSA barriers. Selecting it is COLLECTIVE (window registration); it
  * needs a context with a dist and all ranks in one NVLink domain, else ENCCL (not fatal,
- * the mode is unchanged). Validated on a 1-rank communicator only. */
+ * the mode is unchanged, reason in lmosem_last_error). Its multi-rank logic is validated on
+ * one GPU through the loopback transport below (the same kernel body); NCCL's LSA barriers,
+ * windows and multimem run only on a multi-GPU NVLink node. */
 #define LMOSEM_COMBINE_FUSED 3
 lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode);
+
+/* Emulated world (loopback transport, for tests on ONE GPU). A loopback group of `world`
+ * ranks (1..16) stands in for an NCCL communicator: lmosem_init_loopback creates the
+ * context of one rank on the current device (all ranks of a group on the same device, one
+ * context per rank). The contexts then behave exactly like `world` NCCL ranks — collective
+ * calls (subset_step, reconstruct*, sensitivity) must be made by every rank, each from its
+ * own host thread — and run the same combine code: block split of
+ * the events, the chosen combine (ALLREDUCE / ISD / FUSED; FUSED needs no set-up here), f
+ * replicated. Each collective is NCCL-equivalent: sums over the ranks in rank order, made
+ * by kernels that read the other ranks' buffers behind a host barrier plus stream events.
+ * A rank that does not reach a collective within LMOSEM_TIMEOUT_S seconds (default 300)
+ * fails it with ENCCL on every rank (the group is then broken). The group must outlive its
+ * contexts: lmosem_loopback_destroy returns ESTATE while a context is still registered.
+ * EINVAL: world outside 1..16, NULL pointers, rank outside [0, world), the rank already
+ * taken, or a device other than the group's. */
+typedef struct lmosem_loopback lmosem_loopback;
+lmosem_status lmosem_loopback_create(int32_t world, lmosem_loopback** out);
+lmosem_status lmosem_loopback_destroy(lmosem_loopback* group);
+lmosem_status lmosem_init_loopback(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3],
+                                   const float* norm, lmosem_loopback* group, int32_t rank);
 
 /* The combine mode in effect (-1 for a NULL context). */
 int32_t lmosem_get_combine(const lmosem_ctx* ctx);

@@ -9,10 +9,13 @@
 
 #include <algorithm>
 #include <cerrno>
+#include <chrono>
 #include <cmath>
+#include <condition_variable>
 #include <cstdio>
 #include <cstdlib>
 #include <cstring>
+#include <mutex>
 #include <new>
 #include <string>
 #include <thread>
@@ -21,6 +24,7 @@
 #include "lmosem.h"
 #include "lmosem_kernels.cuh"
 #include "lmosem_fused.cuh"
+#include "lmosem_loop.cuh"
 
 #define LMOSEM_API extern "C" __attribute__((visibility("default")))
 
@@ -34,6 +38,10 @@ struct PhaseMarks {
 
 }  // namespace
 
+#ifndef LMOSEM_FUSED_CTAS_PER_SM
+#define LMOSEM_FUSED_CTAS_PER_SM 4  // fused combine: CTAs (and LSA barriers) per SM
+#endif
+
 // reconstruct_host pipelines the final f download in kPipe brick z-ranges
 constexpr int kPipe = 8;
 // the first subset's upload: kInChunks parts of growing size (1/16, 3/16, 4/16, 8/16 of the
@@ -41,6 +49,27 @@ constexpr int kPipe = 8;
 // first, small part's upload is exposed, and few launches keep their ramp/tail cost low.
 constexpr int kInChunks = 4;
 constexpr int kInChunkEnd[kInChunks + 1] = {0, 1, 4, 8, 16};  // sixteenths of the events
+
+// Loopback group (include/lmosem.h, "Emulated world"): P contexts of one process on one
+// GPU act as P ranks. A collective on rank r is a sequence of phases; each phase boundary
+// records an event on r's stream, waits at the host barrier for all ranks, then makes r's
+// stream wait for every rank's event, so a rank's kernel may read the other ranks' buffers
+// exactly when NCCL's collective would have them ready (lmosem_loop.cuh).
+struct lmosem_loopback {
+    int world = 0;
+    int device = -1;
+    std::mutex m;
+    std::condition_variable cv;
+    int arrived = 0;
+    uint64_t gen = 0;
+    bool broken = false;                 // a rank timed out at a barrier: every later barrier fails
+    std::vector<lmosem_ctx*> ranks;      // registered contexts (nullptr = free slot)
+    std::vector<const float*> src[2];    // per rank: the buffer published at a phase boundary
+                                         // (double-buffered by boundary parity: slot k is rewritten
+                                         // only after every rank has passed the next barrier)
+    unsigned* bar = nullptr;             // fused combine: device barrier counters (one per CTA index)
+    int bar_cap = 0;
+};
 
 struct lmosem_ctx {
     int device = -1;
@@ -66,6 +95,10 @@ struct lmosem_ctx {
     cudaStream_t own_stream = nullptr, stream = nullptr, copy_stream = nullptr;
     int rank = 0, world = 1;
     ncclComm_t comm = nullptr;
+    lmosem_loopback* loop = nullptr;   // loopback transport (test), instead of comm
+    cudaEvent_t loop_ev[2] = {nullptr, nullptr};
+    int loop_phase = 0;
+    const float* loop_peer[lmk::kLoopMax] = {};  // the ranks' buffers published at the last boundary
     bool nccl_mem = false;                          // c, fb from ncclMemAlloc (NVLS-capable)
     void* reg_c = nullptr, * reg_fb = nullptr;       // ncclCommRegister handles
     // fused combine (LMOSEM_COMBINE_FUSED): symmetric windows + device communicator
@@ -229,6 +262,185 @@ int combine_mode(const lmosem_ctx* ctx) {
     return ctx->world > 1 ? LMOSEM_COMBINE_ISD : LMOSEM_COMBINE_ALLREDUCE;
 }
 
+// ------------------------------------------------------------- the combine's transports
+// The collectives of the combine (Listing 3 l.6 copy(add), l.15-16)
+// with NCCL's semantics, through the context's transport: NCCL (one process per GPU) or
+// the loopback group (P contexts on one GPU; test transport). subset_iteration calls only
+// these, so both transports run the same combine code.
+bool has_comm(const lmosem_ctx* ctx) { return ctx->comm != nullptr || ctx->loop != nullptr; }
+
+// seconds a host barrier of the loopback group (and lmosem_synchronize on an NCCL context)
+// waits before declaring the collective failed (LMOSEM_TIMEOUT_S, default 300)
+double coll_timeout_s() {
+    const char* e = std::getenv("LMOSEM_TIMEOUT_S");
+    const double t = e ? std::atof(e) : 300.0;
+    return t > 0 ? t : 300.0;
+}
+
+bool loop_barrier(lmosem_loopback* g) {
+    std::unique_lock<std::mutex> lk(g->m);
+    if (g->broken) return false;
+    const uint64_t my = g->gen;
+    if (++g->arrived == g->world) {
+        g->arrived = 0;
+        ++g->gen;
+        g->cv.notify_all();
+        return true;
+    }
+    const bool ok = g->cv.wait_for(lk, std::chrono::duration<double>(coll_timeout_s()),
+                                   [&] { return g->gen != my || g->broken; });
+    if (!ok || g->broken) {
+        g->broken = true;
+        g->cv.notify_all();
+        return false;
+    }
+    return true;
+}
+
+// Phase boundary of a loopback collective on this rank (see lmosem_loopback): publish
+// `mine` (read by the other ranks until the next boundary), then order this rank's stream
+// after every rank's work so far. Events alternate per boundary, so an event is re-recorded
+// only after every rank has passed the barrier that follows its waits on it.
+lmosem_status loop_boundary(lmosem_ctx* ctx, const float* mine = nullptr) {
+    lmosem_loopback* g = ctx->loop;
+    not_kernel(ctx);
+    const int ph = ctx->loop_phase;
+    CK(cudaEventRecord(ctx->loop_ev[ph], ctx->stream));
+    {
+        std::lock_guard<std::mutex> lk(g->m);
+        g->src[ph][ctx->rank] = mine;
+    }
+    if (!loop_barrier(g))
+        return fail(ctx, LMOSEM_ENCCL, "loopback: a rank did not reach the collective within LMOSEM_TIMEOUT_S");
+    {
+        std::lock_guard<std::mutex> lk(g->m);
+        for (int q = 0; q < ctx->world; ++q) ctx->loop_peer[q] = g->src[ph][q];
+    }
+    for (int q = 0; q < ctx->world; ++q)
+        if (q != ctx->rank) CK(cudaStreamWaitEvent(ctx->stream, g->ranks[q]->loop_ev[ph], 0));
+    ctx->loop_phase ^= 1;
+    return LMOSEM_OK;
+}
+
+lmk::LoopSrc loop_src(const lmosem_ctx* ctx, int64_t add) {
+    lmk::LoopSrc src{};
+    for (int q = 0; q < ctx->world; ++q) src.p[q] = ctx->loop_peer[q] + add;
+    return src;
+}
+
+int loop_grid(const lmosem_ctx* ctx, int64_t n) {
+    return (int)std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, (int64_t)ctx->num_sms * 8));
+}
+
+// recv[i] = sum over ranks of send[rank * count + i], i < count (send == recv - rank * count: in place)
+lmosem_status coll_reduce_scatter(lmosem_ctx* ctx, const float* send, float* recv, size_t count) {
+    if (ctx->comm) {
+        not_kernel(ctx);
+        NK(ncclReduceScatter(send, recv, count, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+        return LMOSEM_OK;
+    }
+    lmosem_status s;
+    if ((s = loop_boundary(ctx, send))) return s;
+    const lmk::LoopSrc src = loop_src(ctx, (int64_t)count * ctx->rank);
+    lmk::k_loop_sum<<<loop_grid(ctx, (int64_t)count), 256, 0, ctx->stream>>>(src, recv, (int64_t)count, ctx->world);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return loop_boundary(ctx);
+}
+
+// recv[rank' * count + i] = send of rank' [i] for every rank' (send == recv + rank * count: in place)
+lmosem_status coll_all_gather(lmosem_ctx* ctx, const float* send, float* recv, size_t count) {
+    if (ctx->comm) {
+        not_kernel(ctx);
+        NK(ncclAllGather(send, recv, count, ncclFloat32, ctx->comm, ctx->stream));
+        return LMOSEM_OK;
+    }
+    lmosem_status s;
+    if ((s = loop_boundary(ctx, send))) return s;
+    lmk::LoopSrc src = loop_src(ctx, 0);
+    for (int q = 0; q <= ctx->world; ++q) src.off[q] = (int64_t)count * q;
+    dim3 grid((unsigned)loop_grid(ctx, (int64_t)count), (unsigned)ctx->world);
+    lmk::k_loop_gather<<<grid, 256, 0, ctx->stream>>>(src, recv, send == recv + (int64_t)count * ctx->rank ? ctx->rank : -1);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return loop_boundary(ctx);
+}
+
+// buf <- sum over ranks of buf (in place), count floats
+lmosem_status coll_all_reduce(lmosem_ctx* ctx, float* buf, size_t count) {
+    if (ctx->comm) {
+        not_kernel(ctx);
+        NK(ncclAllReduce(buf, buf, count, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
+        return LMOSEM_OK;
+    }
+    // reduce-scatter of block r of the count floats into this rank's buf, then all-gather
+    lmk::LoopSrc src{};
+    for (int q = 0; q < ctx->world; ++q) block_range((int64_t)count, q, ctx->world, &src.off[q], &src.off[q + 1]);
+    const int64_t b = src.off[ctx->rank], n = src.off[ctx->rank + 1] - b;
+    lmosem_status s;
+    if ((s = loop_boundary(ctx, buf))) return s;
+    const lmk::LoopSrc part = loop_src(ctx, b);
+    lmk::k_loop_sum<<<loop_grid(ctx, n), 256, 0, ctx->stream>>>(part, buf + b, n, ctx->world);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    if ((s = loop_boundary(ctx, buf))) return s;
+    for (int q = 0; q < ctx->world; ++q) src.p[q] = ctx->loop_peer[q] + src.off[q];
+    dim3 grid((unsigned)loop_grid(ctx, (int64_t)count / ctx->world + 1), (unsigned)ctx->world);
+    lmk::k_loop_gather<<<grid, 256, 0, ctx->stream>>>(src, buf, ctx->rank);
+    CK(cudaGetLastError());
+    ctx->st.launches++;
+    return loop_boundary(ctx);
+}
+
+// The fused ISD combine (NEXT-1; lmosem_fused.cuh): reduce-scatter of c, the block update
+// and the all-gather of f as ONE kernel. NCCL: k_combine_fused over the symmetric windows,
+// a programmatic dependent launch after the projection. Loopback: one cooperative launch
+// of the same body for all ranks (rank 0 launches it between two phase boundaries).
+lmosem_status coll_fused(lmosem_ctx* ctx, int64_t chunk) {
+    if (ctx->comm) {
+        if (ctx->dev_comm_mm)
+            CK(launch_k(ctx, lmk::k_combine_fused<true>, ctx->fused_ctas, 256, 0, ctx->dev_comm, ctx->win_c,
+                        ctx->win_fb, (const float*)ctx->norm, ctx->c, (const float*)ctx->fb, chunk, ctx->bricks.nb,
+                        ctx->bricks));
+        else
+            CK(launch_k(ctx, lmk::k_combine_fused<false>, ctx->fused_ctas, 256, 0, ctx->dev_comm, ctx->win_c,
+                        ctx->win_fb, (const float*)ctx->norm, ctx->c, (const float*)ctx->fb, chunk, ctx->bricks.nb,
+                        ctx->bricks));
+        return LMOSEM_OK;
+    }
+    lmosem_status s;
+    if ((s = loop_boundary(ctx))) return s;
+    if (ctx->rank == 0) {
+        lmosem_loopback* g = ctx->loop;
+        const int P = ctx->world;
+        int per_sm = 0;
+        CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, lmk::k_combine_loop, 256, 0));
+        const int ctas = std::max(1, std::min(LMOSEM_FUSED_CTAS_PER_SM * ctx->num_sms, per_sm * ctx->num_sms / P));
+        if (ctas > g->bar_cap) {
+            if (g->bar) CK(cudaFree(g->bar));
+            g->bar = nullptr;
+            g->bar_cap = 0;
+            CKA(cudaMalloc(&g->bar, sizeof(unsigned) * ctas));
+            g->bar_cap = ctas;
+        }
+        CK(cudaMemsetAsync(g->bar, 0, sizeof(unsigned) * ctas, ctx->stream));
+        lmk::LoopImages im{};
+        for (int q = 0; q < P; ++q) {
+            im.c[q] = g->ranks[q]->c;
+            im.fb[q] = g->ranks[q]->fb;
+            im.s[q] = g->ranks[q]->norm;
+        }
+        unsigned* bar = g->bar;
+        int64_t nb = ctx->bricks.nb;
+        lmk::BrickIt it = ctx->bricks;
+        void* args[] = {&im, &bar, (void*)&P, (void*)&ctas, &chunk, &nb, &it};
+        CK(cudaLaunchCooperativeKernel((const void*)lmk::k_combine_loop, dim3((unsigned)(P * ctas)), dim3(256), args, 0,
+                                       ctx->stream));
+        ctx->st.launches++;
+    }
+    return loop_boundary(ctx);
+}
+
 lmosem_status launch_to_brick(lmosem_ctx* ctx, const float* row, float* br) {
     CK(launch_k(ctx, lmk::k_row_to_brick, grid_for(ctx, ctx->bricks.nb), 256, 0, row, br, ctx->geom, ctx->bricks));
     return LMOSEM_OK;
@@ -254,9 +466,6 @@ int n_slabs(const lmosem_ctx* ctx) {
 
 #ifndef LMOSEM_STATIC_BATCH
 #define LMOSEM_STATIC_BATCH 1  // first claim size from the launch's events per warp
-#endif
-#ifndef LMOSEM_FUSED_CTAS_PER_SM
-#define LMOSEM_FUSED_CTAS_PER_SM 4  // fused combine: CTAs (and LSA barriers) per SM
 #endif
 #ifndef LMOSEM_MIN_BATCH
 #define LMOSEM_MIN_BATCH 4
@@ -425,7 +634,7 @@ lmosem_status get_marks(lmosem_ctx* ctx, PhaseMarks** out) {
 // The final update can be split by brick z-planes (and f downloaded chunk by chunk) only
 // when every rank updates its full replica (no ISD block split).
 bool full_replica_update(const lmosem_ctx* ctx) {
-    return !ctx->comm || combine_mode(ctx) == LMOSEM_COMBINE_ALLREDUCE;
+    return !has_comm(ctx) || combine_mode(ctx) == LMOSEM_COMBINE_ALLREDUCE;
 }
 
 // Host-path pipelining of one subset iteration (reconstruct_host): in_chunks > 1 projects
@@ -462,40 +671,26 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         return s;
     }
     if ((s = mark(ctx, pm, 2))) return s;
-    if (ctx->comm && combine_mode(ctx) == LMOSEM_COMBINE_FUSED && ctx->dev_comm_ok) {
+    if (has_comm(ctx) && combine_mode(ctx) == LMOSEM_COMBINE_FUSED && (ctx->dev_comm_ok || ctx->loop)) {
         // NEXT-1: reduce-scatter + update + all-gather as one kernel over peer memory
-        const int64_t chunk = ctx->nb_alloc / ctx->world;
+        if ((s = coll_fused(ctx, ctx->nb_alloc / ctx->world))) return s;
         if ((s = mark(ctx, pm, 3))) return s;
-        not_kernel(ctx);  // launched plainly: its LSA barriers order it across the ranks
-        if (ctx->dev_comm_mm)
-            lmk::k_combine_fused<true><<<ctx->fused_ctas, 256, 0, ctx->stream>>>(
-                ctx->dev_comm, ctx->win_c, ctx->win_fb, ctx->norm, ctx->c, ctx->fb, chunk, ctx->bricks.nb);
-        else
-            lmk::k_combine_fused<false><<<ctx->fused_ctas, 256, 0, ctx->stream>>>(
-                ctx->dev_comm, ctx->win_c, ctx->win_fb, ctx->norm, ctx->c, ctx->fb, chunk, ctx->bricks.nb);
-        CK(cudaGetLastError());
-        ctx->st.launches++;
         if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
-    } else if (ctx->comm && combine_mode(ctx) == LMOSEM_COMBINE_ISD) {
+    } else if (has_comm(ctx) && combine_mode(ctx) == LMOSEM_COMBINE_ISD) {
         // PAPER.md lines 509-518 (Listing 3 l.15-19): PSD -> ISD. Reduce-scatter c so rank r
         // holds the sum over its brick block, update only that block, all-gather f.
         const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
         int64_t blk_b, blk_e, alloc;
         isd_block(ctx->bricks.nb, ctx->rank, ctx->world, &blk_b, &blk_e, &alloc);
         float* my_c = ctx->c + 8 * b0;
-        not_kernel(ctx);
-        NK(ncclReduceScatter(ctx->c, my_c, (size_t)(8 * chunk), ncclFloat32, ncclSum, ctx->comm, ctx->stream));
-        if ((s = mark(ctx, pm, 3))) return s;
+        if ((s = coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(8 * chunk)))) return s;
         // one launch: the block update (re-zeroes its c) and c <- 0 on every other brick
         if ((s = launch_update(ctx, nullptr, blk_b, blk_e, alloc))) return s;
-        not_kernel(ctx);
-        NK(ncclAllGather(ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk), ncclFloat32, ctx->comm, ctx->stream));
+        if ((s = coll_all_gather(ctx, ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk)))) return s;
+        if ((s = mark(ctx, pm, 3))) return s;
         if (write_f && (s = launch_to_row(ctx, ctx->fb, f, 0))) return s;
     } else {
-        if (ctx->comm) {
-            not_kernel(ctx);
-            NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
-        }
+        if (has_comm(ctx) && (s = coll_all_reduce(ctx, ctx->c, (size_t)ctx->nbf))) return s;
         if ((s = mark(ctx, pm, 3))) return s;
         if (write_f && pipe.host_f) {
             // z-ranges of bricks: bricks [z0, z1) * BX*BY hold rows iz in [2 z0 - 2, 2 z1 - 2)
@@ -595,8 +790,11 @@ LMOSEM_API lmosem_status lmosem_nccl_unique_id(void* out, size_t size) {
     return LMOSEM_OK;
 }
 
-LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3],
-                                     const float* norm, const lmosem_dist* dist) {
+namespace {
+
+// lmosem_init (dist: NCCL communicator) and lmosem_init_loopback (loop: loopback group)
+lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3], const float* norm,
+                       const lmosem_dist* dist, lmosem_loopback* loop, int32_t loop_rank) {
     if (!out) return LMOSEM_EINVAL;
     *out = nullptr;
     if (!dims || !voxel_mm || !norm) return LMOSEM_EINVAL;
@@ -616,6 +814,11 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         world = dist->world;
         if (world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
         if (!dist->nccl_unique_id) return LMOSEM_EINVAL;
+    }
+    if (loop) {
+        rank = loop_rank;
+        world = loop->world;
+        if (rank < 0 || rank >= world) return LMOSEM_EINVAL;
     }
     lmosem_ctx* ctx = new (std::nothrow) lmosem_ctx;
     if (!ctx) return LMOSEM_ENOMEM;
@@ -646,6 +849,7 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     ctx->bricks.BZ = ctx->geom.P[2] / 2;
     ctx->bricks.nb = (int64_t)ctx->bricks.BX * ctx->bricks.BY * ctx->bricks.BZ;
     ctx->nbf = 8 * ctx->bricks.nb;
+    for (int k = 0; k < 3; ++k) ctx->bricks.rhi[k] = (lmk::HALO_LO + dims[k] + 1) / 2;
     {
         int64_t b0, b1;
         isd_block(ctx->bricks.nb, rank, world, &b0, &b1, &ctx->nb_alloc);  // equal ISD brick blocks
@@ -736,6 +940,8 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
         cuda(cudaEventCreateWithFlags(&ctx->ev_consumed[k], cudaEventDisableTiming), "cudaEventCreate");
     }
     for (auto& e : ctx->ev_pipe) cuda(cudaEventCreateWithFlags(&e, cudaEventDisableTiming), "cudaEventCreate");
+    if (loop)
+        for (auto& e : ctx->loop_ev) cuda(cudaEventCreateWithFlags(&e, cudaEventDisableTiming), "cudaEventCreate");
     if (s != LMOSEM_OK) return bail(s);
     cuda(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * V, cudaMemcpyDefault, ctx->stream), "copy norm");
     cuda(cudaMemsetAsync(ctx->c, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream), "memset c");
@@ -770,41 +976,123 @@ LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], co
     }
     cuda(cudaStreamSynchronize(ctx->stream), "sync");
     if (s != LMOSEM_OK) return bail(s);
+    if (loop) {  // join the group: one context per rank, all on the group's device
+        bool joined = false;
+        {
+            std::lock_guard<std::mutex> lk(loop->m);
+            if (loop->device < 0) loop->device = ctx->device;
+            if (loop->device == ctx->device && loop->ranks[rank] == nullptr) {
+                loop->ranks[rank] = ctx;
+                ctx->loop = loop;
+                joined = true;
+            }
+        }
+        if (!joined) {
+            ctx->err = "init_loopback: rank already taken, or a different device than the group's";
+            return bail(LMOSEM_EINVAL);
+        }
+    }
     *out = ctx;
     return LMOSEM_OK;
 }
 
+}  // namespace
+
+LMOSEM_API lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3],
+                                     const float* norm, const lmosem_dist* dist) {
+    return init_ctx(out, dims, voxel_mm, norm, dist, nullptr, 0);
+}
+
+LMOSEM_API lmosem_status lmosem_loopback_create(int32_t world, lmosem_loopback** out) {
+    if (!out) return LMOSEM_EINVAL;
+    *out = nullptr;
+    if (world < 1 || world > lmk::kLoopMax) return LMOSEM_EINVAL;
+    lmosem_loopback* g = new (std::nothrow) lmosem_loopback;
+    if (!g) return LMOSEM_ENOMEM;
+    g->world = world;
+    g->ranks.assign(world, nullptr);
+    g->src[0].assign(world, nullptr);
+    g->src[1].assign(world, nullptr);
+    *out = g;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_loopback_destroy(lmosem_loopback* g) {
+    if (!g) return LMOSEM_OK;
+    {
+        std::lock_guard<std::mutex> lk(g->m);
+        for (auto* c : g->ranks)
+            if (c) return LMOSEM_ESTATE;  // destroy the contexts first
+    }
+    if (g->bar) cudaFree(g->bar);
+    delete g;
+    return LMOSEM_OK;
+}
+
+LMOSEM_API lmosem_status lmosem_init_loopback(lmosem_ctx** out, const int32_t dims[3], const double voxel_mm[3],
+                                              const float* norm, lmosem_loopback* group, int32_t rank) {
+    if (!group) {
+        if (out) *out = nullptr;
+        return LMOSEM_EINVAL;
+    }
+    return init_ctx(out, dims, voxel_mm, norm, nullptr, group, rank);
+}
+
+namespace {
+
+// A status with a message that leaves the context usable (unlike fail() for ENCCL/ECUDA).
+lmosem_status soft_fail(lmosem_ctx* ctx, lmosem_status s, const std::string& msg) {
+    ctx->err = msg;
+    return s;
+}
+
+// Collective set-up of the fused combine over NCCL: symmetric windows over c and the brick
+// f, and a device communicator with one LSA barrier per CTA of the fused kernel (multimem
+// when the team has it). On failure everything registered here is released again and the
+// context stays usable (ENCCL with the reason in lmosem_last_error).
+lmosem_status setup_fused(lmosem_ctx* ctx) {
+    if (!ctx->comm || !ctx->nccl_mem)
+        return soft_fail(ctx, LMOSEM_ENCCL, "set_combine(FUSED): needs a context with a dist and ncclMemAlloc images");
+    CK(cudaStreamSynchronize(ctx->stream));
+    const size_t bytes = sizeof(float) * 8 * ctx->nb_alloc;
+    auto undo = [&](const std::string& why, ncclResult_t r) {
+        if (ctx->win_c) ncclCommWindowDeregister(ctx->comm, ctx->win_c);
+        if (ctx->win_fb) ncclCommWindowDeregister(ctx->comm, ctx->win_fb);
+        ctx->win_c = ctx->win_fb = nullptr;
+        return soft_fail(ctx, LMOSEM_ENCCL, "set_combine(FUSED): " + why + (r != ncclSuccess ? std::string(": ") + ncclGetErrorString(r) : ""));
+    };
+    ncclResult_t r = ncclCommWindowRegister(ctx->comm, ctx->c, bytes, &ctx->win_c, NCCL_WIN_COLL_SYMMETRIC);
+    if (r != ncclSuccess) return (ctx->win_c = nullptr, undo("ncclCommWindowRegister(c)", r));
+    r = ncclCommWindowRegister(ctx->comm, ctx->fb, bytes, &ctx->win_fb, NCCL_WIN_COLL_SYMMETRIC);
+    if (r != ncclSuccess) return (ctx->win_fb = nullptr, undo("ncclCommWindowRegister(fb)", r));
+    ctx->fused_ctas = LMOSEM_FUSED_CTAS_PER_SM * ctx->num_sms;  // all co-resident (barrier per CTA)
+    ncclDevCommRequirements reqs;
+    std::memset(&reqs, 0, sizeof(reqs));
+    reqs.lsaBarrierCount = ctx->fused_ctas;
+    reqs.lsaMultimem = ctx->world > 1;
+    r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
+    if (r != ncclSuccess && reqs.lsaMultimem) {
+        reqs.lsaMultimem = false;
+        r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
+    }
+    if (r != ncclSuccess) return undo("ncclDevCommCreate", r);
+    if (ctx->dev_comm.lsaSize != ctx->world) {  // not one NVLink domain: keep the NCCL collectives
+        ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
+        return undo("the ranks are not one NVLink (LSA) domain", ncclSuccess);
+    }
+    ctx->dev_comm_ok = true;
+    ctx->dev_comm_mm = reqs.lsaMultimem;
+    return LMOSEM_OK;
+}
+
+}  // namespace
+
 LMOSEM_API lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode) {
     USABLE(ctx);
     if (mode < 0 || mode > LMOSEM_COMBINE_FUSED) return fail(ctx, LMOSEM_EINVAL, "set_combine: bad mode");
-    if (mode == LMOSEM_COMBINE_FUSED && !ctx->dev_comm_ok) {
-        // collective: symmetric windows over c and the brick f, and a device communicator
-        // with one LSA barrier per CTA of the fused kernel (multimem when the team has it)
-        if (!ctx->comm || !ctx->nccl_mem)
-            return LMOSEM_ENCCL;  // needs a communicator and NCCL-allocated images (not fatal)
-        CK(cudaStreamSynchronize(ctx->stream));
-        const size_t bytes = sizeof(float) * 8 * ctx->nb_alloc;
-        if (!ctx->win_c && ncclCommWindowRegister(ctx->comm, ctx->c, bytes, &ctx->win_c, NCCL_WIN_COLL_SYMMETRIC) != ncclSuccess)
-            return (ctx->win_c = nullptr, LMOSEM_ENCCL);
-        if (!ctx->win_fb && ncclCommWindowRegister(ctx->comm, ctx->fb, bytes, &ctx->win_fb, NCCL_WIN_COLL_SYMMETRIC) != ncclSuccess)
-            return (ctx->win_fb = nullptr, LMOSEM_ENCCL);
-        ctx->fused_ctas = LMOSEM_FUSED_CTAS_PER_SM * ctx->num_sms;  // all co-resident (barrier per CTA)
-        ncclDevCommRequirements reqs;
-        std::memset(&reqs, 0, sizeof(reqs));
-        reqs.lsaBarrierCount = ctx->fused_ctas;
-        reqs.lsaMultimem = ctx->world > 1;
-        ncclResult_t r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
-        if (r != ncclSuccess && reqs.lsaMultimem) {
-            reqs.lsaMultimem = false;
-            r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
-        }
-        if (r != ncclSuccess) return LMOSEM_ENCCL;
-        if (ctx->dev_comm.lsaSize != ctx->world) {  // not one NVLink domain: keep the NCCL collectives
-            ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
-            return LMOSEM_ENCCL;
-        }
-        ctx->dev_comm_ok = true;
-        ctx->dev_comm_mm = reqs.lsaMultimem;
+    if (mode == LMOSEM_COMBINE_FUSED && !ctx->dev_comm_ok && !ctx->loop) {
+        lmosem_status s = setup_fused(ctx);
+        if (s) return s;
     }
     ctx->combine = mode;
     return LMOSEM_OK;
@@ -1100,10 +1388,7 @@ LMOSEM_API lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event*
     block_range(n_events, ctx->rank, ctx->world, &b, &e);
     lmosem_status s;
     if ((s = launch_project(ctx, events + b, e - b, nullptr, 4))) return s;
-    if (ctx->comm) {
-        not_kernel(ctx);
-        NK(ncclAllReduce(ctx->c, ctx->c, (size_t)ctx->nbf, ncclFloat32, ncclSum, ctx->comm, ctx->stream));
-    }
+    if (has_comm(ctx) && (s = coll_all_reduce(ctx, ctx->c, (size_t)ctx->nbf))) return s;
     return launch_to_row(ctx, ctx->c, s_out, 1);  // s_out <- c, c <- 0
 }
 
@@ -1180,6 +1465,12 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
         ctx->c = ctx->fb = nullptr;
     }
     if (ctx->comm) ncclCommDestroy(ctx->comm);
+    if (ctx->loop) {
+        std::lock_guard<std::mutex> lk(ctx->loop->m);
+        ctx->loop->ranks[ctx->rank] = nullptr;
+    }
+    for (auto e : ctx->loop_ev)
+        if (e) cudaEventDestroy(e);
     for (auto& pm : ctx->pending)
         for (int k = 0; k < 5; ++k) cudaEventDestroy(pm.e[k]);
     for (auto& pm : ctx->pool)

@@ -8,10 +8,18 @@
 //   -> barrier (CTA k of every rank done) -> each CTA re-zeroes, in its local c, exactly
 //      the bricks CTA k read on every rank (the LSA barrier orders CTA k across ranks,
 //      not the CTAs of one rank, so no CTA may touch bricks another CTA still reads).
-// Replaces reduce-scatter + update + all-gather; NVLink bytes per GPU with multimem are
-// ~2*|c|/P instead of ~2*(P-1)/P*|c|. Opt-in (LMOSEM_COMBINE_FUSED): with one GPU per test
-// call only the 1-rank NCCL peer-pointer path can run here; the body (combine_fused_body in
-// lmosem_kernels.cuh) is also run with 2-8 emulated ranks on one GPU (tests/cuda/combine_emu.cu).
+// Replaces reduce-scatter + update + all-gather by one kernel. NVLink bytes per GPU: the
+// NVSwitch still pulls every rank's partial c of the block, so each GPU's egress for the
+// reduce is ~(P-1)/P*|c| (23.6 MB of the 27 MB brick c at P = 8, >= 31 us at the ~770 GB/s
+// peer rate); what multimem saves is the all-gather egress (one multimem.st per brick
+// instead of P-1 stores) and the overlap of egress with ingress in one pass. Halo-only
+// bricks (6.5 % of the C2 image) are not exchanged. Launched as a programmatic dependent
+// launch after the projection (pdl_wait before the first barrier) and triggering its own
+// dependents at once, so the next subset's k_project can claim events and run its float64
+// setup during the combine (every CTA of this kernel is resident before any dependent CTA).
+// The multi-rank logic runs on one GPU through the loopback transport (lmosem_loop.cuh,
+// the same body with P emulated ranks); NCCL's LSA barrier, windows and multimem only on
+// a multi-GPU node.
 #pragma once
 #include <cuda/atomic>
 #include <nccl.h>
@@ -108,9 +116,12 @@ struct NcclTeam {
 template <bool MM>
 __global__ void __launch_bounds__(256) k_combine_fused(ncclDevComm dc, ncclWindow_t wc, ncclWindow_t wf,
                                                        const float* __restrict__ sb, float* __restrict__ c_local,
-                                                       const float* __restrict__ fb_local, int64_t chunk, int64_t nb) {
+                                                       const float* __restrict__ fb_local, int64_t chunk, int64_t nb,
+                                                       BrickIt it) {
+    pdl_wait();     // the projection of every CTA of this rank is complete
+    pdl_trigger();  // all CTAs of this kernel are resident: the next kernel may start its prologue
     NcclTeam<MM> team{dc, wc, wf};
-    combine_fused_body(team, blockIdx.x, gridDim.x, sb, c_local, fb_local, chunk, nb);
+    combine_fused_body(team, blockIdx.x, gridDim.x, sb, c_local, fb_local, chunk, nb, it);
 }
 
 }  // namespace lmk

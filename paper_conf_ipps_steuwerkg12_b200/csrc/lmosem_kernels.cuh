@@ -596,7 +596,19 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
 struct BrickIt {
     int BX, BY, BZ;
     int64_t nb;
+    int rhi[3];  // bricks [HALO_LO/2, rhi[k]) of axis k hold real voxels (0: no halo skipping)
 };
+
+// A brick with at least one real voxel (the fused combine skips halo-only bricks: their f
+// stays 0 and nothing reads their c).
+__device__ __forceinline__ bool real_brick(const BrickIt& it, int64_t b) {
+    if (it.rhi[0] == 0) return true;
+    const unsigned u = (unsigned)b, bx = u % (unsigned)it.BX, t = u / (unsigned)it.BX;
+    const unsigned by = t % (unsigned)it.BY, bz = t / (unsigned)it.BY;
+    constexpr unsigned lo = HALO_LO / 2;
+    return bx >= lo && bx < (unsigned)it.rhi[0] && by >= lo && by < (unsigned)it.rhi[1] && bz >= lo &&
+           bz < (unsigned)it.rhi[2];
+}
 
 __device__ __forceinline__ bool real_voxel(const GridGeom& g, int px, int py, int pz, int64_t& r) {
     const int ix = px - HALO_LO, iy = py - HALO_LO, iz = pz - HALO_LO;
@@ -721,27 +733,38 @@ __device__ __forceinline__ float4 upd4(float4 f, float4 c, float4 s) {
 template <class T>
 __device__ __forceinline__ void combine_fused_body(T team, int cta, int ctas, const float* __restrict__ sb,
                                                    float* __restrict__ c_local, const float* __restrict__ fb_local,
-                                                   int64_t chunk, int64_t nb) {
+                                                   int64_t chunk, int64_t nb, const BrickIt& it) {
     team.sync(cta);  // every rank's projection has finished writing its c
     const int nr = team.size();
     const int64_t b0 = chunk * team.rank(), b1 = b0 + chunk < nb ? b0 + chunk : nb;
     const int64_t t0 = (int64_t)cta * blockDim.x + threadIdx.x, stride = (int64_t)ctas * blockDim.x;
-    // two bricks per thread per iteration: their c sums are in flight together
+    // two bricks per thread per iteration: their c sums are in flight together; halo-only
+    // bricks are skipped (no exchange)
     int64_t b = b0 + t0;
     for (; b + stride < b1; b += 2 * stride) {
+        const bool ra = real_brick(it, b), rb = real_brick(it, b + stride);
         const size_t oa = (size_t)b * 32, ob = (size_t)(b + stride) * 32;
-        float4 ca0, ca1, cb0, cb1;
-        team.sum_c2(oa, ob, ca0, ca1, cb0, cb1);
         const float4* Fa = reinterpret_cast<const float4*>(fb_local + 8 * b);
         const float4* Fb = reinterpret_cast<const float4*>(fb_local + 8 * (b + stride));
         const float4* Sa = reinterpret_cast<const float4*>(sb + 8 * b);
         const float4* Sb = reinterpret_cast<const float4*>(sb + 8 * (b + stride));
-        const float4 na0 = upd4(Fa[0], ca0, __ldg(Sa)), na1 = upd4(Fa[1], ca1, __ldg(Sa + 1));
-        const float4 nb0 = upd4(Fb[0], cb0, __ldg(Sb)), nb1 = upd4(Fb[1], cb1, __ldg(Sb + 1));
-        team.store_f(oa, na0, na1);
-        team.store_f(ob, nb0, nb1);
+        if (ra && rb) {
+            float4 ca0, ca1, cb0, cb1;
+            team.sum_c2(oa, ob, ca0, ca1, cb0, cb1);
+            const float4 na0 = upd4(Fa[0], ca0, __ldg(Sa)), na1 = upd4(Fa[1], ca1, __ldg(Sa + 1));
+            const float4 nb0 = upd4(Fb[0], cb0, __ldg(Sb)), nb1 = upd4(Fb[1], cb1, __ldg(Sb + 1));
+            team.store_f(oa, na0, na1);
+            team.store_f(ob, nb0, nb1);
+        } else if (ra || rb) {
+            const size_t off = ra ? oa : ob;
+            const float4* F = ra ? Fa : Fb;
+            const float4* S = ra ? Sa : Sb;
+            float4 c0, c1;
+            team.sum_c(off, c0, c1);
+            team.store_f(off, upd4(F[0], c0, __ldg(S)), upd4(F[1], c1, __ldg(S + 1)));
+        }
     }
-    if (b < b1) {
+    if (b < b1 && real_brick(it, b)) {
         const size_t off = (size_t)b * 32;
         float4 c0, c1;
         team.sum_c(off, c0, c1);
@@ -752,7 +775,8 @@ __device__ __forceinline__ void combine_fused_body(T team, int cta, int ctas, co
     }
     team.sync(cta);  // CTA k of every rank has read its bricks of every c and written f
     // re-zero, in the local c, exactly the bricks CTA k read on every rank (the barrier
-    // orders CTA k across ranks, not the CTAs of one rank)
+    // orders CTA k across ranks, not the CTAs of one rank); halo-only bricks too (rounding
+    // slivers of step 1 may have added to them; nobody reads them)
     float4* C = reinterpret_cast<float4*>(c_local);
     const float4 z = make_float4(0.f, 0.f, 0.f, 0.f);
     for (int q = 0; q < nr; ++q) {

@@ -27,7 +27,8 @@ EXPORTS = (
     "lmosem_forward", "lmosem_update", "lmosem_synchronize", "lmosem_set_timing", "lmosem_get_stats",
     "lmosem_destroy", "lmosem_last_error", "lmosem_set_slabs", "lmosem_get_slabs",
     "lmosem_sensitivity", "lmosem_set_norm", "lmosem_set_combine", "lmosem_get_combine",
-    "lmosem_reconstruct_file", "lmosem_isd_block",
+    "lmosem_reconstruct_file", "lmosem_isd_block", "lmosem_loopback_create", "lmosem_loopback_destroy",
+    "lmosem_init_loopback",
 )
 COMBINE_ALLREDUCE, COMBINE_ISD, COMBINE_FUSED = 1, 2, 3
 
@@ -75,6 +76,9 @@ def load(build_if_missing: bool = False) -> ctypes.CDLL:
         "lmosem_isd_block": ([_I64, _I32, _I32, ctypes.POINTER(_I64), ctypes.POINTER(_I64), ctypes.POINTER(_I64)], _S),
         "lmosem_nccl_unique_id": ([_P, ctypes.c_size_t], _S),
         "lmosem_init": ([ctypes.POINTER(_P), _P, _P, _P, ctypes.POINTER(Dist)], _S),
+        "lmosem_loopback_create": ([_I32, ctypes.POINTER(_P)], _S),
+        "lmosem_loopback_destroy": ([_P], _S),
+        "lmosem_init_loopback": ([ctypes.POINTER(_P), _P, _P, _P, _P, _I32], _S),
         "lmosem_set_stream": ([_P, _P], _S),
         "lmosem_set_slabs": ([_P, _I32], _S),
         "lmosem_set_combine": ([_P, _I32], _S),
@@ -162,15 +166,45 @@ def _host_ptr(a, numel: int | None = None) -> int:
     return a.ctypes.data
 
 
+class Loopback:
+    """An emulated world of `world` ranks on one GPU (include/lmosem.h, "Emulated world"):
+    pass ``loopback=(group, rank)`` to Reconstructor, one context per rank, and drive each
+    rank's collective calls from its own thread. Test transport: the contexts run the same
+    combine code as NCCL ranks. Close the contexts before the group."""
+
+    def __init__(self, world: int):
+        self._lib = load()
+        h = _P()
+        st = self._lib.lmosem_loopback_create(int(world), ctypes.byref(h))
+        if st != OK:
+            raise LmosemError(st, f"loopback_create({world})")
+        self._h = h
+        self.world = int(world)
+
+    def close(self):
+        if getattr(self, "_h", None) is not None and self._h.value:
+            st = self._lib.lmosem_loopback_destroy(self._h)
+            if st != OK:
+                raise LmosemError(st, "loopback_destroy: contexts still registered")
+            self._h = _P()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
 class Reconstructor:
     """One LM-OSEM context (one GPU / rank). See include/lmosem.h for semantics.
 
     ``norm``: V float32 sensitivity image (CUDA tensor or host array), copied at init.
     ``dist``: None for one GPU, or (rank, world, nccl_id_bytes) for a collective context.
     ``stream``: torch.cuda.Stream to enqueue on (default: torch's current stream).
+    ``loopback``: (Loopback, rank) for a rank of an emulated world on this GPU (tests).
     """
 
-    def __init__(self, dims, voxel_mm, norm, dist=None, stream=None):
+    def __init__(self, dims, voxel_mm, norm, dist=None, stream=None, loopback=None):
         import torch
         lib = load()
         if not torch.cuda.is_available():
@@ -193,11 +227,21 @@ class Reconstructor:
             self._keep = ctypes.create_string_buffer(bytes(uid), NCCL_ID_BYTES)
             dptr = ctypes.byref(Dist(int(rank), int(world), ctypes.cast(self._keep, ctypes.c_void_p)))
         h = _P()
-        st = lib.lmosem_init(ctypes.byref(h), d, v, nptr, dptr)
+        if dist is not None and loopback is not None:
+            raise ValueError("dist and loopback are exclusive")
+        if loopback is not None:
+            group, rank = loopback
+            self._group = group  # the group outlives this context
+            st = lib.lmosem_init_loopback(ctypes.byref(h), d, v, nptr, group._h, int(rank))
+        else:
+            st = lib.lmosem_init(ctypes.byref(h), d, v, nptr, dptr)
         if st != OK:
             raise LmosemError(st, lib.lmosem_last_error(None).decode())
         self._h = h
-        self.rank, self.world = (0, 1) if dist is None else (int(dist[0]), int(dist[1]))
+        if loopback is not None:
+            self.rank, self.world = int(loopback[1]), loopback[0].world
+        else:
+            self.rank, self.world = (0, 1) if dist is None else (int(dist[0]), int(dist[1]))
         self.set_stream(stream if stream is not None else torch.cuda.current_stream())
 
     # -- plumbing

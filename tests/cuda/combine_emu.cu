@@ -56,7 +56,7 @@ __global__ void __launch_bounds__(256) k_emu(float* const* c, float* const* f, f
                                              int ctas, int64_t chunk, int64_t nb) {
     const int r = blockIdx.x / ctas, k = blockIdx.x % ctas;
     EmuTeam team{c, f, bar, r, P, 0u};
-    lmk::combine_fused_body(team, k, ctas, s[r], c[r], f[r], chunk, nb);
+    lmk::combine_fused_body(team, k, ctas, s[r], c[r], f[r], chunk, nb, lmk::BrickIt{});
 }
 
 static unsigned lcg(unsigned& x) { return x = x * 1664525u + 1013904223u; }

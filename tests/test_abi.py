@@ -156,3 +156,21 @@ def test_l2peak_exports_and_rejects_bad_arguments(lib):
     ms, ops = ctypes.c_float(), ctypes.c_double()
     for mode, n, k in [(7, 1 << 20, 4), (-1, 1 << 20, 4), (0, 10, 4), (0, 1 << 20, 0), (0, 1 << 33, 4)]:
         assert l2.l2peak_run(mode, n, k, ctypes.byref(ms), ctypes.byref(ops)) == -1
+
+
+def test_loopback_group_arguments(lib):
+    """The loopback group (include/lmosem.h "Emulated world"): world 1..16, NULL checks and
+    rank range before any CUDA call; destroy of an empty group and of NULL is OK."""
+    h = ctypes.c_void_p()
+    for bad in (0, -1, 17):
+        assert lib.lmosem_loopback_create(bad, ctypes.byref(h)) == L.EINVAL and not h.value
+    assert lib.lmosem_loopback_create(2, None) == L.EINVAL
+    assert lib.lmosem_loopback_create(2, ctypes.byref(h)) == L.OK and h.value
+    c = ctypes.c_void_p(123)
+    d = (ctypes.c_int32 * 3)(4, 4, 4)
+    v = (ctypes.c_double * 3)(1, 1, 1)
+    for rank in (-1, 2):
+        assert lib.lmosem_init_loopback(ctypes.byref(c), d, v, 1, h, rank) == L.EINVAL and not c.value
+    assert lib.lmosem_init_loopback(ctypes.byref(c), d, v, 1, None, 0) == L.EINVAL
+    assert lib.lmosem_loopback_destroy(h) == L.OK
+    assert lib.lmosem_loopback_destroy(None) == L.OK
