@@ -18,6 +18,7 @@
  *    the half-open box [x0+ix*vx, x0+(ix+1)*vx) x ..., x0 = -nx*vx/2; images are float32
  *    with linear index j = ix + nx*(iy + ny*iz) (x fastest). V = nx*ny*nz < 2^31.
  *  - Event: lmosem_event, 6 float32 (two detection points in mm, the segment p1 -> p2).
+ *    Device event arrays must be 8-byte aligned (EINVAL otherwise).
  *    Non-finite, zero-length or volume-missing events, and events with fp_i <= 0,
  *    contribute nothing (not an error).
  *  - Pointers: "device" = CUDA device memory of the context's device; "host" = host
@@ -138,14 +139,18 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  *     l.15-19): ncclReduceScatter(c) gives rank r the sum over its contiguous block of the
  *     internal image, rank r updates only that block (1/P of step 2), ncclAllGather
  *     rebuilds the full f on every rank. Same NVLink bytes, 1/P of the update work.
- * 0 (default) = ISD when world > 1, else ALLREDUCE. EINVAL for other values. */
+ * 0 (default) = FUSED when world > 1 over NCCL, the LSA team has multimem (NVLS) and the
+ * fused kernel passed its self-test at init (set LMOSEM_AUTO_FUSED=0 to skip it); else ISD
+ * when world > 1; else ALLREDUCE. EINVAL for other values. */
 #define LMOSEM_COMBINE_ALLREDUCE 1
 #define LMOSEM_COMBINE_ISD 2
 /* LMOSEM_COMBINE_FUSED (opt-in): the ISD switch as ONE kernel over
  * NVLink peer memory (NCCL 2.28 symmetric windows + device communicator): rank r reads its
  * block of c summed over ranks (multimem.ld_reduce in the NVSwitch when available, else
  * peer loads), updates it and writes the new f block to every rank (multimem.st or peer
- * stores), between two LSA barriers. Selecting it is COLLECTIVE (window registration); it
+ * stores), between two LSA barriers. Setting it up runs a self-test of the kernel on a known
+ * pattern on every rank (verdict agreed over the communicator; failure = ENCCL, the NCCL
+ * collectives stay in use). Selecting it is COLLECTIVE (window registration); it
  * needs a context with a dist and all ranks in one NVLink domain, else ENCCL (not fatal,
  * the mode is unchanged, reason in lmosem_last_error). Its multi-rank logic is validated on
  * one GPU through the loopback transport below (the same kernel body); NCCL's LSA barriers,
@@ -246,7 +251,11 @@ lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm);
  * both V float32 x-fastest; the context's norm); c is re-zeroed. */
 lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c);
 
-/* Waits for all work enqueued by this context. Reports asynchronous kernel faults. */
+/* Waits for all work enqueued by this context. Reports asynchronous kernel faults. With an
+ * NCCL communicator it is a watchdog: ncclCommGetAsyncError is polled, and after
+ * LMOSEM_TIMEOUT_S seconds (default 300) without completion — a peer rank that died or never
+ * reached the collective — the communicator is aborted and ENCCL returned (the context then
+ * answers ESTATE). The synchronous host/file reconstructions wait the same way. */
 lmosem_status lmosem_synchronize(lmosem_ctx* ctx);
 
 /* Enables (1) / disables (0) per-phase CUDA-event timing; enabling clears the times. */

@@ -2,6 +2,7 @@
 // LM-OSEM subset iteration (§IV, Listings 2-3). Kernels: lmosem_kernels.cuh.
 #include <cuda_runtime.h>
 #include <nccl.h>
+#include <nvtx3/nvToolsExt.h>
 
 #include <fcntl.h>
 #include <sys/stat.h>
@@ -81,6 +82,7 @@ struct lmosem_ctx {
     int64_t nbf = 0;           // floats per padded brick image (8 * bricks)
     int64_t nb_alloc = 0;      // bricks allocated: nb rounded up to a multiple of world
     int combine = 0;           // LMOSEM_COMBINE_* (0 = auto)
+    int auto_combine = 0;      // the auto mode: FUSED when multimem set up and self-tested at init, else ISD (world > 1)
     float* c = nullptr;        // error image, bricks (kept all-zero between subsets)
     float* fb = nullptr;       // brick copy of the current f
     float* norm = nullptr;     // s in bricks (halo = 0)
@@ -123,6 +125,8 @@ struct lmosem_ctx {
     std::vector<Occ> occ;      // k_project residency per (mode, path-buffer bytes)
     bool failed = false;
     std::string err;
+    int debug_stall_ms = 0;    // LMOSEM_DEBUG_STALL_MS (tests of the watchdog): a stall before each combine
+    int* abort_flag = nullptr; // host-mapped; raised by abort_comm (polled by k_debug_stall)
     // timing
     bool timing = false;
     std::vector<PhaseMarks> pending, pool;
@@ -166,6 +170,11 @@ bool device_accessible(const void* p) {
 bool device_accessible(const void* a, const void* b, const void* c = nullptr) {
     return device_accessible(a) && device_accessible(b) && device_accessible(c);
 }
+
+// The event loaders read 8-byte (float2) or, for 16-byte aligned tiles, 16-byte vectors: an
+// event array must be 8-byte aligned (every event then is: 24 B records). A misaligned
+// pointer is EINVAL before anything is enqueued instead of a kernel fault.
+bool events_misaligned(const void* ev, int64_t n) { return n > 0 && ((uintptr_t)ev & 7u) != 0; }
 
 #define CK(call)                                                                                    \
     do {                                                                                            \
@@ -221,6 +230,18 @@ cudaError_t launch_k(lmosem_ctx* ctx, void (*kernel)(KArgs...), int grid, int bl
     return e;
 }
 
+// LMOSEM_DEBUG_STALL_MS: a bounded spin of `ns` nanoseconds standing in for a peer that is
+// late to the combine (tests of the watchdog in wait_done; never set in production). Like
+// NCCL's own kernels it also polls an abort flag (host-mapped), which abort_comm raises.
+__global__ void k_debug_stall(unsigned long long ns, const volatile int* abort_flag) {
+    unsigned long long t0, t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t0));
+    do {
+        __nanosleep(100000);
+        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    } while (t - t0 < ns && *abort_flag == 0);
+}
+
 // any operation on ctx->stream that is not one of the library's kernels
 inline void not_kernel(lmosem_ctx* ctx) { ctx->after_kernel = false; }
 
@@ -259,6 +280,7 @@ int grid_for(lmosem_ctx* ctx, int64_t items) {
 
 int combine_mode(const lmosem_ctx* ctx) {
     if (ctx->combine) return ctx->combine;
+    if (ctx->auto_combine) return ctx->auto_combine;
     return ctx->world > 1 ? LMOSEM_COMBINE_ISD : LMOSEM_COMBINE_ALLREDUCE;
 }
 
@@ -609,6 +631,65 @@ lmosem_status launch_update(lmosem_ctx* ctx, float* f_row, int64_t b_begin = 0, 
     return LMOSEM_OK;
 }
 
+// NVTX range over one phase of a subset iteration (host enqueue side; nsys correlates the
+// launches inside it). Costs a few ns without a tool attached.
+struct Nvtx {
+    explicit Nvtx(const char* name) { nvtxRangePushA(name); }
+    void next(const char* name) {  // closes this range and opens the next phase's
+        nvtxRangePop();
+        nvtxRangePushA(name);
+    }
+    ~Nvtx() { nvtxRangePop(); }
+};
+
+// After a failed or timed-out collective: abort the communicator so NCCL kernels stuck on
+// a dead peer exit, and forget every handle tied to it (the context is then failed).
+void abort_comm(lmosem_ctx* ctx) {
+    if (!ctx->comm) return;
+    if (ctx->abort_flag) *(volatile int*)ctx->abort_flag = 1;
+    ncclCommAbort(ctx->comm);
+    ctx->comm = nullptr;
+    ctx->dev_comm_ok = false;
+    ctx->win_c = ctx->win_fb = nullptr;
+    ctx->reg_c = ctx->reg_fb = nullptr;
+}
+
+// Waits until `ev` (or, with ev == nullptr, stream `st`) completes. With an NCCL
+// communicator this is a watchdog: it polls ncclCommGetAsyncError and gives up after
+// LMOSEM_TIMEOUT_S seconds (a peer that died or never joined the collective), aborting the
+// communicator; the result is ENCCL and the context answers ESTATE from then on.
+lmosem_status wait_done(lmosem_ctx* ctx, cudaStream_t st, cudaEvent_t ev = nullptr) {
+    if (!ctx->comm) {
+        CK(ev ? cudaEventSynchronize(ev) : cudaStreamSynchronize(st));
+        return LMOSEM_OK;
+    }
+    const auto t0 = std::chrono::steady_clock::now();
+    const double limit = coll_timeout_s();
+    for (;;) {
+        const cudaError_t e = ev ? cudaEventQuery(ev) : cudaStreamQuery(st);
+        if (e == cudaSuccess) return LMOSEM_OK;
+        if (e != cudaErrorNotReady) {
+            abort_comm(ctx);
+            return fail(ctx, LMOSEM_ECUDA, std::string("wait: ") + cudaGetErrorString(e));
+        }
+        ncclResult_t ae = ncclSuccess;
+        const ncclResult_t r = ncclCommGetAsyncError(ctx->comm, &ae);
+        if (r != ncclSuccess || (ae != ncclSuccess && ae != ncclInProgress)) {
+            const std::string why = ncclGetErrorString(r != ncclSuccess ? r : ae);
+            abort_comm(ctx);
+            return fail(ctx, LMOSEM_ENCCL, "nccl async error: " + why + " (communicator aborted)");
+        }
+        const double waited = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
+        if (waited > limit) {
+            abort_comm(ctx);
+            return fail(ctx, LMOSEM_ENCCL, "timed out after " + std::to_string((int)limit) +
+                                               " s (LMOSEM_TIMEOUT_S) waiting for the stream: a peer rank stalled "
+                                               "or died; communicator aborted");
+        }
+        std::this_thread::sleep_for(std::chrono::microseconds(50));
+    }
+}
+
 lmosem_status mark(lmosem_ctx* ctx, PhaseMarks* pm, int k) {
     if (pm) {
         not_kernel(ctx);
@@ -651,6 +732,7 @@ struct HostPipe {
 // to_brick: refresh ctx->fb from f first; write_f: write the updated f to the caller.
 lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n, float* f, bool whole_subset,
                                bool to_brick, bool write_f, const HostPipe& pipe = HostPipe()) {
+    Nvtx range_subset("lmosem subset");
     int64_t b = 0, e = n;
     if (whole_subset) block_range(n, ctx->rank, ctx->world, &b, &e);
     PhaseMarks* pm = nullptr;
@@ -659,6 +741,7 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
     if ((s = mark(ctx, pm, 0))) return s;
     if (to_brick && (s = launch_to_brick(ctx, f, ctx->fb))) return s;
     if ((s = mark(ctx, pm, 1))) return s;
+    Nvtx range_project("lmosem project");  // then the combine + update
     if (pipe.in_chunks > 1) {
         for (int q = 0; q < pipe.in_chunks; ++q) {
             int64_t qb, qe;
@@ -671,6 +754,12 @@ lmosem_status subset_iteration(lmosem_ctx* ctx, const lmosem_event* ev, int64_t 
         return s;
     }
     if ((s = mark(ctx, pm, 2))) return s;
+    range_project.next("lmosem combine + update");
+    if (has_comm(ctx) && ctx->debug_stall_ms > 0) {  // tests of the watchdog only
+        not_kernel(ctx);
+        k_debug_stall<<<1, 32, 0, ctx->stream>>>(1000000ull * (unsigned long long)ctx->debug_stall_ms, ctx->abort_flag);
+        CK(cudaGetLastError());
+    }
     if (has_comm(ctx) && combine_mode(ctx) == LMOSEM_COMBINE_FUSED && (ctx->dev_comm_ok || ctx->loop)) {
         // NEXT-1: reduce-scatter + update + all-gather as one kernel over peer memory
         if ((s = coll_fused(ctx, ctx->nb_alloc / ctx->world))) return s;
@@ -729,7 +818,8 @@ lmosem_status check_offsets(const int64_t* off, int32_t L) {
 
 lmosem_status resolve_timing(lmosem_ctx* ctx) {
     for (auto& pm : ctx->pending) {
-        CK(cudaEventSynchronize(pm.e[4]));
+        lmosem_status ws = wait_done(ctx, nullptr, pm.e[4]);
+        if (ws) return ws;
         float t[4];
         for (int k = 0; k < 4; ++k) CK(cudaEventElapsedTime(&t[k], pm.e[k], pm.e[k + 1]));
         ctx->st.convert_ms += t[0];
@@ -741,7 +831,8 @@ lmosem_status resolve_timing(lmosem_ctx* ctx) {
     }
     ctx->pending.clear();
     for (size_t k = 0; k + 1 < ctx->h2d_pending.size(); k += 2) {
-        CK(cudaEventSynchronize(ctx->h2d_pending[k + 1]));
+        lmosem_status ws = wait_done(ctx, nullptr, ctx->h2d_pending[k + 1]);
+        if (ws) return ws;
         float t;
         CK(cudaEventElapsedTime(&t, ctx->h2d_pending[k], ctx->h2d_pending[k + 1]));
         ctx->st.h2d_ms += t;
@@ -789,6 +880,111 @@ LMOSEM_API lmosem_status lmosem_nccl_unique_id(void* out, size_t size) {
     std::memcpy(out, &id, sizeof(id));
     return LMOSEM_OK;
 }
+
+namespace {
+
+// A status with a message that leaves the context usable (unlike fail() for ENCCL/ECUDA).
+lmosem_status soft_fail(lmosem_ctx* ctx, lmosem_status s, const std::string& msg) {
+    ctx->err = msg;
+    return s;
+}
+
+// Runs the fused combine once on the k_selftest_fill pattern (collective) and agrees on the
+// verdict over the communicator (max of the mismatch counts); c and the brick f are zero
+// again afterwards (f is refreshed from the caller's image at the next subset).
+lmosem_status fused_selftest(lmosem_ctx* ctx, bool* passed) {
+    *passed = false;
+    const int64_t nbf_alloc = 8 * ctx->nb_alloc;
+    float* ones = nullptr;
+    int* bad = nullptr;
+    CKA(cudaMalloc(&ones, sizeof(float) * nbf_alloc));
+    if (cudaMalloc(&bad, sizeof(int)) != cudaSuccess) {
+        cudaFree(ones);
+        (void)cudaGetLastError();
+        return fail(ctx, LMOSEM_ENOMEM, "fused self-test: cudaMalloc");
+    }
+    const float P = (float)ctx->world;
+    lmosem_status s = LMOSEM_OK;
+    float* norm = ctx->norm;
+    ctx->norm = ones;  // the fused kernel reads the context's norm: s = 1 for the test
+    int h_bad = -1;
+    do {
+        not_kernel(ctx);
+        if (cudaMemsetAsync(bad, 0, sizeof(int), ctx->stream) != cudaSuccess) { s = fail(ctx, LMOSEM_ECUDA, "self-test memset"); break; }
+        lmk::k_selftest_fill<<<grid_for(ctx, nbf_alloc), 256, 0, ctx->stream>>>(ctx->c, ctx->fb, ones, nbf_alloc,
+                                                                                (float)(ctx->rank + 1));
+        if ((s = coll_fused(ctx, ctx->nb_alloc / ctx->world))) break;
+        lmk::k_selftest_check<<<grid_for(ctx, ctx->bricks.nb), 256, 0, ctx->stream>>>(ctx->c, ctx->fb, ctx->bricks,
+                                                                                       0.5f * P * (P + 1.0f), bad);
+        not_kernel(ctx);
+        if (ncclAllReduce(bad, bad, 1, ncclInt32, ncclMax, ctx->comm, ctx->stream) != ncclSuccess) {
+            s = fail(ctx, LMOSEM_ENCCL, "fused self-test: ncclAllReduce");
+            break;
+        }
+        if (cudaMemcpyAsync(&h_bad, bad, sizeof(int), cudaMemcpyDeviceToHost, ctx->stream) != cudaSuccess ||
+            cudaMemsetAsync(ctx->c, 0, sizeof(float) * nbf_alloc, ctx->stream) != cudaSuccess ||
+            cudaMemsetAsync(ctx->fb, 0, sizeof(float) * nbf_alloc, ctx->stream) != cudaSuccess) {
+            s = fail(ctx, LMOSEM_ECUDA, "fused self-test: copy");
+            break;
+        }
+        s = wait_done(ctx, ctx->stream);
+    } while (false);
+    ctx->norm = norm;
+    cudaFree(ones);
+    cudaFree(bad);
+    if (s) return s;
+    *passed = h_bad == 0;
+    return LMOSEM_OK;
+}
+
+// Collective set-up of the fused combine over NCCL: symmetric windows over c and the brick
+// f, and a device communicator with one LSA barrier per CTA of the fused kernel (multimem
+// when the team has it). On failure everything registered here is released again and the
+// context stays usable (ENCCL with the reason in lmosem_last_error).
+lmosem_status setup_fused(lmosem_ctx* ctx) {
+    if (!ctx->comm || !ctx->nccl_mem)
+        return soft_fail(ctx, LMOSEM_ENCCL, "set_combine(FUSED): needs a context with a dist and ncclMemAlloc images");
+    CK(cudaStreamSynchronize(ctx->stream));
+    const size_t bytes = sizeof(float) * 8 * ctx->nb_alloc;
+    auto undo = [&](const std::string& why, ncclResult_t r) {
+        if (ctx->win_c) ncclCommWindowDeregister(ctx->comm, ctx->win_c);
+        if (ctx->win_fb) ncclCommWindowDeregister(ctx->comm, ctx->win_fb);
+        ctx->win_c = ctx->win_fb = nullptr;
+        return soft_fail(ctx, LMOSEM_ENCCL, "set_combine(FUSED): " + why + (r != ncclSuccess ? std::string(": ") + ncclGetErrorString(r) : ""));
+    };
+    ncclResult_t r = ncclCommWindowRegister(ctx->comm, ctx->c, bytes, &ctx->win_c, NCCL_WIN_COLL_SYMMETRIC);
+    if (r != ncclSuccess) return (ctx->win_c = nullptr, undo("ncclCommWindowRegister(c)", r));
+    r = ncclCommWindowRegister(ctx->comm, ctx->fb, bytes, &ctx->win_fb, NCCL_WIN_COLL_SYMMETRIC);
+    if (r != ncclSuccess) return (ctx->win_fb = nullptr, undo("ncclCommWindowRegister(fb)", r));
+    ctx->fused_ctas = LMOSEM_FUSED_CTAS_PER_SM * ctx->num_sms;  // all co-resident (barrier per CTA)
+    ncclDevCommRequirements reqs;
+    std::memset(&reqs, 0, sizeof(reqs));
+    reqs.lsaBarrierCount = ctx->fused_ctas;
+    reqs.lsaMultimem = ctx->world > 1;
+    r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
+    if (r != ncclSuccess && reqs.lsaMultimem) {
+        reqs.lsaMultimem = false;
+        r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
+    }
+    if (r != ncclSuccess) return undo("ncclDevCommCreate", r);
+    if (ctx->dev_comm.lsaSize != ctx->world) {  // not one NVLink domain: keep the NCCL collectives
+        ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
+        return undo("the ranks are not one NVLink (LSA) domain", ncclSuccess);
+    }
+    ctx->dev_comm_ok = true;
+    ctx->dev_comm_mm = reqs.lsaMultimem;
+    bool passed = false;
+    lmosem_status s = fused_selftest(ctx, &passed);
+    if (s) return s;
+    if (!passed) {
+        ctx->dev_comm_ok = ctx->dev_comm_mm = false;
+        ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
+        return undo("self-test on the known pattern failed (kept the NCCL collectives)", ncclSuccess);
+    }
+    return LMOSEM_OK;
+}
+
+}  // namespace
 
 namespace {
 
@@ -883,6 +1079,12 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (!cuda(cudaGetDeviceProperties(&prop, ctx->device), "cudaGetDeviceProperties")) return bail(s);
     ctx->num_sms = prop.multiProcessorCount;
     if (const char* e = std::getenv("LMOSEM_PDL")) ctx->pdl = e[0] != '0';  // A/B switch (default on)
+    if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
+    if (ctx->debug_stall_ms > 0) {
+        if (!cuda(cudaHostAlloc(&ctx->abort_flag, sizeof(int), cudaHostAllocMapped), "cudaHostAlloc(abort flag)"))
+            return bail(s);
+        *ctx->abort_flag = 0;
+    }
     if (ctx->proj_smem > (size_t)prop.sharedMemPerBlockOptin) {
         ctx->err = "volume too large for the shared-memory path buffer";
         return bail(LMOSEM_EINVAL);
@@ -976,6 +1178,17 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     }
     cuda(cudaStreamSynchronize(ctx->stream), "sync");
     if (s != LMOSEM_OK) return bail(s);
+    // world > 1 over NCCL: set up the fused combine (NEXT-1) and self-test it; it becomes the
+    // automatic combine when the LSA team has multimem (NVLS). Otherwise, or with
+    // LMOSEM_AUTO_FUSED=0, the automatic combine is ISD (reduce-scatter + all-gather).
+    if (ctx->comm && world > 1) {
+        const char* af = std::getenv("LMOSEM_AUTO_FUSED");
+        if (!(af && af[0] == '0')) {
+            const lmosem_status fs = setup_fused(ctx);
+            if (ctx->failed) return bail(fs);
+            if (fs == LMOSEM_OK && ctx->dev_comm_mm) ctx->auto_combine = LMOSEM_COMBINE_FUSED;
+        }
+    }
     if (loop) {  // join the group: one context per rank, all on the group's device
         bool joined = false;
         {
@@ -1038,54 +1251,6 @@ LMOSEM_API lmosem_status lmosem_init_loopback(lmosem_ctx** out, const int32_t di
     return init_ctx(out, dims, voxel_mm, norm, nullptr, group, rank);
 }
 
-namespace {
-
-// A status with a message that leaves the context usable (unlike fail() for ENCCL/ECUDA).
-lmosem_status soft_fail(lmosem_ctx* ctx, lmosem_status s, const std::string& msg) {
-    ctx->err = msg;
-    return s;
-}
-
-// Collective set-up of the fused combine over NCCL: symmetric windows over c and the brick
-// f, and a device communicator with one LSA barrier per CTA of the fused kernel (multimem
-// when the team has it). On failure everything registered here is released again and the
-// context stays usable (ENCCL with the reason in lmosem_last_error).
-lmosem_status setup_fused(lmosem_ctx* ctx) {
-    if (!ctx->comm || !ctx->nccl_mem)
-        return soft_fail(ctx, LMOSEM_ENCCL, "set_combine(FUSED): needs a context with a dist and ncclMemAlloc images");
-    CK(cudaStreamSynchronize(ctx->stream));
-    const size_t bytes = sizeof(float) * 8 * ctx->nb_alloc;
-    auto undo = [&](const std::string& why, ncclResult_t r) {
-        if (ctx->win_c) ncclCommWindowDeregister(ctx->comm, ctx->win_c);
-        if (ctx->win_fb) ncclCommWindowDeregister(ctx->comm, ctx->win_fb);
-        ctx->win_c = ctx->win_fb = nullptr;
-        return soft_fail(ctx, LMOSEM_ENCCL, "set_combine(FUSED): " + why + (r != ncclSuccess ? std::string(": ") + ncclGetErrorString(r) : ""));
-    };
-    ncclResult_t r = ncclCommWindowRegister(ctx->comm, ctx->c, bytes, &ctx->win_c, NCCL_WIN_COLL_SYMMETRIC);
-    if (r != ncclSuccess) return (ctx->win_c = nullptr, undo("ncclCommWindowRegister(c)", r));
-    r = ncclCommWindowRegister(ctx->comm, ctx->fb, bytes, &ctx->win_fb, NCCL_WIN_COLL_SYMMETRIC);
-    if (r != ncclSuccess) return (ctx->win_fb = nullptr, undo("ncclCommWindowRegister(fb)", r));
-    ctx->fused_ctas = LMOSEM_FUSED_CTAS_PER_SM * ctx->num_sms;  // all co-resident (barrier per CTA)
-    ncclDevCommRequirements reqs;
-    std::memset(&reqs, 0, sizeof(reqs));
-    reqs.lsaBarrierCount = ctx->fused_ctas;
-    reqs.lsaMultimem = ctx->world > 1;
-    r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
-    if (r != ncclSuccess && reqs.lsaMultimem) {
-        reqs.lsaMultimem = false;
-        r = ncclDevCommCreate(ctx->comm, &reqs, &ctx->dev_comm);
-    }
-    if (r != ncclSuccess) return undo("ncclDevCommCreate", r);
-    if (ctx->dev_comm.lsaSize != ctx->world) {  // not one NVLink domain: keep the NCCL collectives
-        ncclDevCommDestroy(ctx->comm, &ctx->dev_comm);
-        return undo("the ranks are not one NVLink (LSA) domain", ncclSuccess);
-    }
-    ctx->dev_comm_ok = true;
-    ctx->dev_comm_mm = reqs.lsaMultimem;
-    return LMOSEM_OK;
-}
-
-}  // namespace
 
 LMOSEM_API lmosem_status lmosem_set_combine(lmosem_ctx* ctx, int32_t mode) {
     USABLE(ctx);
@@ -1120,6 +1285,7 @@ LMOSEM_API lmosem_status lmosem_subset_step(lmosem_ctx* ctx, const lmosem_event*
     if (!f || n_events < 0 || (n_events > 0 && !events)) return fail(ctx, LMOSEM_EINVAL, "subset_step: bad arguments");
     if (!device_accessible(f, n_events > 0 ? events : nullptr))
         return fail(ctx, LMOSEM_EINVAL, "subset_step: events / f are not device-accessible memory");
+    if (events_misaligned(events, n_events)) return fail(ctx, LMOSEM_EINVAL, "subset_step: events not 8-byte aligned");
     return subset_iteration(ctx, events, n_events, f, true, true, true);
 }
 
@@ -1130,6 +1296,8 @@ LMOSEM_API lmosem_status lmosem_reconstruct(lmosem_ctx* ctx, const lmosem_event*
         return fail(ctx, LMOSEM_EINVAL, "reconstruct: bad arguments");
     if (!device_accessible(f, offsets[n_subsets] > offsets[0] ? events : nullptr))
         return fail(ctx, LMOSEM_EINVAL, "reconstruct: events / f are not device-accessible memory");
+    if (events_misaligned(events, offsets[n_subsets] - offsets[0]))
+        return fail(ctx, LMOSEM_EINVAL, "reconstruct: events not 8-byte aligned");
     const int64_t total = (int64_t)n_iterations * n_subsets;
     int64_t step = 0;
     for (int32_t it = 0; it < n_iterations; ++it)
@@ -1251,10 +1419,7 @@ LMOSEM_API lmosem_status lmosem_reconstruct_file(lmosem_ctx* ctx, const char* pa
             int64_t b, e;
             block_range(offsets[l + 1] - offsets[l], ctx->rank, ctx->world, &b, &e);
             // host: read this rank's block while the GPU works on the previous subset
-            if (cudaEventSynchronize(ctx->ev_copied[k]) != cudaSuccess) {
-                s = fail(ctx, LMOSEM_ECUDA, "reconstruct_file: staging sync");
-                break;
-            }
+            if ((s = wait_done(ctx, nullptr, ctx->ev_copied[k]))) break;
             if (e > b && !pread_parallel(fd, ctx->pin_ev[k], sizeof(lmosem_event) * (e - b),
                                          (off_t)(sizeof(lmosem_event) * (offsets[l] + b)))) {
                 s = fail(ctx, LMOSEM_EIO, std::string("reconstruct_file: read ") + path + ": " + strerror(errno));
@@ -1274,10 +1439,14 @@ LMOSEM_API lmosem_status lmosem_reconstruct_file(lmosem_ctx* ctx, const char* pa
                 s = fail(ctx, LMOSEM_ECUDA, "reconstruct_file: cudaEventRecord");
         }
     close(fd);
-    if (s == LMOSEM_EIO) cudaStreamSynchronize(ctx->stream);  // nothing left in flight on return
+    if (s == LMOSEM_EIO) {  // nothing left in flight on return
+        const std::string msg = ctx->err;
+        lmosem_status ws = wait_done(ctx, ctx->stream);
+        if (ws) return ws;
+        ctx->err = msg;
+    }
     if (s) return s;
-    CK(cudaStreamSynchronize(ctx->stream));
-    return LMOSEM_OK;
+    return wait_done(ctx, ctx->stream);
 }
 
 LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_event* events, const int64_t* offsets,
@@ -1347,9 +1516,9 @@ LMOSEM_API lmosem_status lmosem_reconstruct_host(lmosem_ctx* ctx, const lmosem_e
         }
     if (!pipe_out || total == 0)
         CK(cudaMemcpyAsync(f, ctx->dev_f, sizeof(float) * ctx->V, cudaMemcpyDeviceToHost, ctx->stream));
-    CK(cudaStreamSynchronize(ctx->stream));
-    CK(cudaStreamSynchronize(ctx->copy_stream));
-    return LMOSEM_OK;
+    lmosem_status ws = wait_done(ctx, ctx->stream);
+    if (ws) return ws;
+    return wait_done(ctx, ctx->copy_stream);
 }
 
 LMOSEM_API lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event* events, int64_t n_events,
@@ -1359,6 +1528,7 @@ LMOSEM_API lmosem_status lmosem_error_image(lmosem_ctx* ctx, const lmosem_event*
         return fail(ctx, LMOSEM_EINVAL, "error_image: bad arguments");
     if (!device_accessible(f, c_out, n_events > 0 ? events : nullptr))
         return fail(ctx, LMOSEM_EINVAL, "error_image: buffers are not device-accessible memory");
+    if (events_misaligned(events, n_events)) return fail(ctx, LMOSEM_EINVAL, "error_image: events not 8-byte aligned");
     lmosem_status s;
     if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
     if ((s = launch_project(ctx, events, n_events, nullptr, 0))) return s;
@@ -1372,6 +1542,7 @@ LMOSEM_API lmosem_status lmosem_forward(lmosem_ctx* ctx, const lmosem_event* eve
         return fail(ctx, LMOSEM_EINVAL, "forward: bad arguments");
     if (!device_accessible(f, n_events > 0 ? events : nullptr, n_events > 0 ? fp_out : nullptr))
         return fail(ctx, LMOSEM_EINVAL, "forward: buffers are not device-accessible memory");
+    if (events_misaligned(events, n_events)) return fail(ctx, LMOSEM_EINVAL, "forward: events not 8-byte aligned");
     lmosem_status s;
     if ((s = launch_to_brick(ctx, f, ctx->fb))) return s;
     return launch_project(ctx, events, n_events, fp_out, 1);
@@ -1384,6 +1555,7 @@ LMOSEM_API lmosem_status lmosem_sensitivity(lmosem_ctx* ctx, const lmosem_event*
         return fail(ctx, LMOSEM_EINVAL, "sensitivity: bad arguments");
     if (!device_accessible(s_out, n_events > 0 ? events : nullptr))
         return fail(ctx, LMOSEM_EINVAL, "sensitivity: buffers are not device-accessible memory");
+    if (events_misaligned(events, n_events)) return fail(ctx, LMOSEM_EINVAL, "sensitivity: events not 8-byte aligned");
     int64_t b = 0, e = n_events;
     block_range(n_events, ctx->rank, ctx->world, &b, &e);
     lmosem_status s;
@@ -1398,8 +1570,7 @@ LMOSEM_API lmosem_status lmosem_set_norm(lmosem_ctx* ctx, const float* norm) {
     CK(cudaMemcpyAsync(ctx->scratch, norm, sizeof(float) * ctx->V, cudaMemcpyDefault, ctx->stream));
     lmosem_status s = launch_to_brick(ctx, ctx->scratch, ctx->norm);
     if (s) return s;
-    CK(cudaStreamSynchronize(ctx->stream));  // the caller may release `norm` on return
-    return LMOSEM_OK;
+    return wait_done(ctx, ctx->stream);  // the caller may release `norm` on return
 }
 
 LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {
@@ -1416,13 +1587,16 @@ LMOSEM_API lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c) {
 
 LMOSEM_API lmosem_status lmosem_synchronize(lmosem_ctx* ctx) {
     USABLE(ctx);
-    CK(cudaStreamSynchronize(ctx->stream));
-    CK(cudaStreamSynchronize(ctx->copy_stream));
+    lmosem_status s = wait_done(ctx, ctx->stream);
+    if (s) return s;
+    if ((s = wait_done(ctx, ctx->copy_stream))) return s;
     if (ctx->comm) {
         ncclResult_t async_err = ncclSuccess;
         NK(ncclCommGetAsyncError(ctx->comm, &async_err));
-        if (async_err != ncclSuccess)
+        if (async_err != ncclSuccess) {
+            abort_comm(ctx);
             return fail(ctx, LMOSEM_ENCCL, std::string("nccl async: ") + ncclGetErrorString(async_err));
+        }
     }
     return LMOSEM_OK;
 }
@@ -1486,6 +1660,7 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     for (auto e : ctx->ev_pipe)
         if (e) cudaEventDestroy(e);
     if (ctx->dev_f) cudaFree(ctx->dev_f);
+    if (ctx->abort_flag) cudaFreeHost(ctx->abort_flag);
     if (ctx->geom.tex_fb) cudaDestroyTextureObject(ctx->geom.tex_fb);
     if (ctx->c) cudaFree(ctx->c);
     if (ctx->fb) cudaFree(ctx->fb);

@@ -124,4 +124,27 @@ __global__ void __launch_bounds__(256) k_combine_fused(ncclDevComm dc, ncclWindo
     combine_fused_body(team, blockIdx.x, gridDim.x, sb, c_local, fb_local, chunk, nb, it);
 }
 
+// Self-test of the fused combine on a known pattern (run once when it is set up, on every
+// rank, before it may become the default): c = rank + 1, brick f = 1, s = 1 on every brick;
+// afterwards every real brick must hold f = sum_q (q + 1) = P(P+1)/2 (exact in float32),
+// every halo-only brick f = 1, and c = 0 everywhere.
+__global__ void __launch_bounds__(256) k_selftest_fill(float* __restrict__ c, float* __restrict__ fb,
+                                                       float* __restrict__ s, int64_t nbf, float cval) {
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nbf; i += (int64_t)gridDim.x * blockDim.x) {
+        c[i] = cval;
+        fb[i] = 1.0f;
+        s[i] = 1.0f;
+    }
+}
+
+__global__ void __launch_bounds__(256) k_selftest_check(const float* __restrict__ c, const float* __restrict__ fb,
+                                                        BrickIt it, float expect, int* __restrict__ bad) {
+    int nbad = 0;
+    for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < it.nb; b += (int64_t)gridDim.x * blockDim.x) {
+        const float e = real_brick(it, b) ? expect : 1.0f;
+        for (int q = 0; q < 8; ++q) nbad += (fb[8 * b + q] != e) + (c[8 * b + q] != 0.0f);
+    }
+    if (nbad) atomicAdd(bad, nbad);
+}
+
 }  // namespace lmk

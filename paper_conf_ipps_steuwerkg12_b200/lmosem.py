@@ -284,16 +284,28 @@ class Reconstructor:
         ep, n = self._events_ptr(events)
         self._check(self._lib.lmosem_subset_step(self._h, ep, n, _dev_ptr(f, "float32", self.V)))
 
+    @staticmethod
+    def _offsets(offsets, n: int) -> np.ndarray:
+        """Subset offsets as int64; the C side cannot see the event count, so the binding
+        checks that every subset lies inside the n events it was given."""
+        off = np.ascontiguousarray(offsets, dtype=np.int64)
+        if off.ndim != 1 or off.size < 1:
+            raise ValueError("offsets must be a 1-D array of n_subsets + 1 entries")
+        if off[0] < 0 or off[-1] > n or np.any(np.diff(off) < 0):
+            raise ValueError(f"offsets must be non-decreasing within [0, {n}]")
+        return off
+
     def reconstruct(self, events, offsets, n_iterations, f):
         """n_iterations passes over subsets events[offsets[l]:offsets[l+1]] (in events)."""
-        ep, _ = self._events_ptr(events)
-        off = np.ascontiguousarray(offsets, dtype=np.int64)
+        ep, n = self._events_ptr(events)
+        off = self._offsets(offsets, n)
         self._check(self._lib.lmosem_reconstruct(self._h, ep, off.ctypes.data, off.size - 1, int(n_iterations),
                                                  _dev_ptr(f, "float32", self.V)))
 
     def reconstruct_host(self, events, offsets, n_iterations, f):
         """Host events + host f (in/out); H2D streaming overlapped with projection."""
-        off = np.ascontiguousarray(offsets, dtype=np.int64)
+        n = (events.numel() if hasattr(events, "numel") else np.asarray(events).size) // 6
+        off = self._offsets(offsets, n)
         self._check(self._lib.lmosem_reconstruct_host(self._h, _host_ptr(events), off.ctypes.data, off.size - 1,
                                                       int(n_iterations), _host_ptr(f, self.V)))
 

@@ -568,9 +568,11 @@ def test_user_stream_and_argument_errors(pkg):
     ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, np.ones(cfg.n_voxels))
     assert rel_l2(f2.cpu().numpy().astype(np.float64), ref) <= REL_L2_RECON
     for bad_off, iters in [(off[::-1].copy(), 1), (off - 5, 1), (off, -1)]:
-        with pytest.raises(pkg.LmosemError) as e:
+        with pytest.raises((pkg.LmosemError, ValueError)):  # the binding checks offsets first
             rec.reconstruct(evd, bad_off, iters, f)
-        assert e.value.status == 1
+        o = np.ascontiguousarray(bad_off, np.int64)  # the C side's own check (EINVAL)
+        assert rec._lib.lmosem_reconstruct(rec._h, evd.data_ptr(), o.ctypes.data, o.size - 1, iters,
+                                           f.data_ptr()) == 1
     g0 = f.clone()
     rec.reconstruct(evd, off, 0, f)  # zero iterations: f unchanged
     rec.synchronize()
@@ -809,3 +811,55 @@ def test_lsu_and_texture_gathers(pkg, monkeypatch, tex):
     ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 1, s, f0.astype(np.float64))
     assert maxrel(got, ref) <= 2 * MAXREL_SUBSET
     assert rel_l2(got, ref) <= REL_L2_RECON
+
+
+def test_misaligned_events_and_bad_offsets_rejected(pkg):
+    """A device event array that is not 8-byte aligned is EINVAL before any launch (not a
+    kernel fault), and the binding rejects subset offsets outside the events it was given;
+    the context stays usable after both."""
+    import ctypes
+    cfg, ev, s = inputs("C1")
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    buf = dev(np.concatenate([[0.0], ev[:100].ravel()]).astype(np.float32))  # events at +4 B
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    lib = pkg.load()
+    st = lib.lmosem_subset_step(rec._h, ctypes.c_void_p(buf.data_ptr() + 4), 100, ctypes.c_void_p(f.data_ptr()))
+    assert st == 1  # EINVAL
+    with pytest.raises(ValueError):
+        rec.reconstruct(dev(ev[:100]), [0, 50, 101], 1, f)
+    with pytest.raises(ValueError):
+        rec.reconstruct_host(ev[:100], [0, 60, 40], 1, np.ones(cfg.n_voxels, np.float32))
+    rec.subset_step(dev(ev[:cfg.n_events]), f)
+    rec.synchronize()
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], s, np.ones(cfg.n_voxels))
+    assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
+    rec.close()
+
+
+def test_watchdog_aborts_stalled_combine(pkg, monkeypatch):
+    """SURVEY.md §5 failure detection: a combine that does not finish (here a debug stall
+    of 4 s in front of the NCCL collective, standing in for a dead peer) makes
+    lmosem_synchronize return ENCCL about 1 s (NCCL's abort) after LMOSEM_TIMEOUT_S instead
+    of hanging (the stall, like NCCL's kernels, polls the abort flag); the
+    communicator is aborted and the context answers ESTATE afterwards."""
+    import time
+    monkeypatch.setenv("LMOSEM_TIMEOUT_S", "1")
+    monkeypatch.setenv("LMOSEM_DEBUG_STALL_MS", "4000")
+    cfg, ev, s = inputs("C1")
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), dist=(0, 1, pkg.nccl_unique_id()))
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    d_ev = dev(ev[:cfg.n_events])
+    torch.cuda.synchronize()
+    rec.subset_step(d_ev, f)
+    t0 = time.time()
+    with pytest.raises(pkg.LmosemError) as e:
+        rec.synchronize()
+    waited = time.time() - t0
+    print(f"[watchdog] synchronize returned after {waited:.2f} s (timeout 1 s + ncclCommAbort)")
+    # measured on B200: ~2.0 s = the 1 s timeout + ~1 s of NCCL's own ncclCommAbort teardown
+    assert e.value.status in (3, 4) and waited < 2.5, (e.value, waited)  # ECUDA / ENCCL
+    assert "LMOSEM_TIMEOUT_S" in str(e.value) or "nccl" in str(e.value)
+    with pytest.raises(pkg.LmosemError) as e2:
+        rec.subset_step(d_ev, f)
+    assert e2.value.status == 5  # ESTATE
+    rec.close()

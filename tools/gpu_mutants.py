@@ -4,7 +4,7 @@ plausible kernel bug, are built here (`build`, nvcc cross-compiles) and run on t
 (`run`) against a fast subset of tests/test_parity_gpu.py with LMOSEM_LIB pointing at the
 mutant. A mutant the parity tests do not catch is reported as SURVIVED (diagnostic; the
 results are in profiles/r01_gpu_mutants.txt).
-Usage: python tools/gpu_mutants.py build | run"""
+Usage: python tools/gpu_mutants.py build|run [name-substring]"""
 import json
 import os
 import shutil
@@ -60,6 +60,24 @@ MUTANTS = [
      "            dep_ready = true;", False),
     ("z-slab boundaries off by one brick", H, "g.clo[2] = 2 * (int)((int64_t)half * k / K);",
      "g.clo[2] = 2 * (int)((int64_t)half * k / K) + (k > 0 ? 2 : 0);", False),
+    # the multi-rank combine (round 2: caught by tests/test_loopback_gpu.py, P ranks on one GPU)
+    ("combine: events not block-split (every rank projects the whole subset)", H,
+     "if (whole_subset) block_range(n, ctx->rank, ctx->world, &b, &e);", "if (false) block_range(n, ctx->rank, ctx->world, &b, &e);", False),
+    ("combine: ISD block offset ignores the rank", H, "b0 = chunk * ctx->rank;", "b0 = 0;", False),
+    ("combine: reduce-scatter count in bricks, not floats", H, "coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(8 * chunk))",
+     "coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(chunk))", False),
+    ("combine: ISD update leaves the other ranks' partial c (no zero_to)", H,
+     "launch_update(ctx, nullptr, blk_b, blk_e, alloc)", "launch_update(ctx, nullptr, blk_b, blk_e)", False),
+    ("combine: ISD all-gather of f dropped", H,
+     "        if ((s = coll_all_gather(ctx, ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk)))) return s;\n", "", False),
+    ("combine: all-reduce over a brick count", H, "coll_all_reduce(ctx, ctx->c, (size_t)ctx->nbf)",
+     "coll_all_reduce(ctx, ctx->c, (size_t)ctx->bricks.nb)", True),
+    ("fused combine: every rank takes rank 0's block", K, "const int64_t b0 = chunk * team.rank(), b1",
+     "const int64_t b0 = chunk * 0, b1", False),
+    ("fused combine: the last real brick column treated as halo", K, "bx < (unsigned)it.rhi[0]",
+     "bx + 1 < (unsigned)it.rhi[0]", False),
+    ("fused combine: local c not re-zeroed", K, "            C[2 * b] = z;\n            C[2 * b + 1] = z;\n", "", False),
+    ("fused combine: second brick of a pair not stored", K, "            team.store_f(ob, nb0, nb1);\n", "", False),
 ]
 # Not listed: equivalent mutants. Dropping the 2^-40 offset of the mirrored frame changes
 # only exactly integral up-moving positions, where "voxel m - 1 with a crossing at d = 0"
@@ -69,16 +87,22 @@ MUTANTS = [
 # covered by the gloo tests and the emulated-rank combine test). The z-slab pass B setup
 # test `ok && fp_known > 0` only saves work: the back-projection's own fp > 0 guard skips
 # the same events (measured: the mutant passes every parity test, as expected).
-TESTS = ("golden or degenerate or axis_parallel or c1_ or zslab_passes_match_oracle_c1 or odd_extents or "
+TESTS = ("loopback_c1 or loopback_c2 or loopback_ragged or golden or degenerate or axis_parallel or c1_ or zslab_passes_match_oracle_c1 or odd_extents or "
          "lors_in_voxel_faces or one_subset_paper_shaped or programmatic or nccl_combine_single_rank or "
          "combine_modes_single_rank or zero_forward_projection or lsu_and_texture")
 
 
-def build():
+def _selected(name, only):
+    return only is None or name == "control" or only in name
+
+
+def build(only=None):
     from paper_conf_ipps_steuwerkg12_b200 import build as b
     os.makedirs(OUT, exist_ok=True)
     names = [("control", None, None, None, False)] + MUTANTS
     for i, (name, fn, old, new, every) in enumerate(names):
+        if not _selected(name, only):
+            continue
         d = os.path.join(OUT, f"src{i}")
         shutil.rmtree(d, ignore_errors=True)
         shutil.copytree(CSRC, d)
@@ -92,12 +116,15 @@ def build():
         print("built", i, name, flush=True)
 
 
-def run():
+def run(only=None):
     names = [("control", None, None, None, False)] + MUTANTS
     res = []
     for i, (name, *_rest) in enumerate(names):
+        if not _selected(name, only):
+            continue
         env = dict(os.environ, LMOSEM_LIB=os.path.join(OUT, f"liblmosem_m{i}.so"))
-        out = subprocess.run([sys.executable, "-m", "pytest", os.path.join(ROOT, "tests", "test_parity_gpu.py"), "-x",
+        out = subprocess.run([sys.executable, "-m", "pytest", os.path.join(ROOT, "tests", "test_parity_gpu.py"),
+                              os.path.join(ROOT, "tests", "test_loopback_gpu.py"), "-x",
                               "-q", "-p", "no:cacheprovider", "-k", TESTS], capture_output=True, text=True, cwd=ROOT,
                              env=env, timeout=900)
         tail = [ln for ln in out.stdout.splitlines() if ln.startswith("FAILED") or " passed" in ln or " failed" in ln]
@@ -109,4 +136,4 @@ def run():
 
 
 if __name__ == "__main__":
-    {"build": build, "run": run}[sys.argv[1]]()
+    {"build": build, "run": run}[sys.argv[1]](sys.argv[2] if len(sys.argv) > 2 else None)
