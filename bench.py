@@ -39,6 +39,9 @@ METRIC = "LM-OSEM events/s per subset (150x150x280)"
 # (tools/path_stats.py, oracle on a 20k-event sample)
 MEAN_PATH = {"C1": 25.37, "C2": 252.19, "C3": 252.19, "C4": 506.79, "C5": 440.96}
 FLUSH_BYTES = 256 << 20
+# NVLink 5 unidirectional GPU-to-GPU rate used to MODEL the combine's floor (t_AR,roof in
+# SURVEY.md §8(d)); not measured here: every run of this repo has one GPU
+NVLINK_GBS = 770.0
 # The paper's own runtimes, as context only (Fig. 4b):
 # the bar heights did not survive text extraction
 PAPER_CONTEXT = {
@@ -71,7 +74,8 @@ def parse():
     ap.add_argument("--e2e-file", action="store_true",
                     help="also time lmosem_reconstruct_file from a raw list-mode file (page cache)")
     ap.add_argument("--combine", default="auto", choices=["auto", "allreduce", "isd", "fused"],
-                    help="combine of the per-GPU error images for N > 1 (default: isd)")
+                    help="combine of the per-GPU error images for N > 1 (default: the library's auto mode, "
+                         "fused when NVLS multimem is available and self-tested, else isd)")
     return ap.parse_args()
 
 
@@ -146,7 +150,8 @@ def l2_peak_gbs(V: int, nbf: int):
     lib.l2peak_run.argtypes = [ctypes.c_int, ctypes.c_int64, ctypes.c_int32, ctypes.POINTER(ctypes.c_float),
                                ctypes.POINTER(ctypes.c_double)]
     out = {}
-    for name, mode in (("red", 0), ("ldg", 1), ("pair", 2), ("pair_run8", 4), ("pair_warp32", 5)):
+    for name, mode in (("red", 0), ("ldg", 1), ("pair", 2), ("pair_run8", 4), ("pair_warp32", 5),
+                       ("ldg_warp32", 7), ("red_warp32", 8)):
         ms, ops = ctypes.c_float(), ctypes.c_double()
         if lib.l2peak_run(mode, V, 256, ctypes.byref(ms), ctypes.byref(ops)) != 0:
             return None
@@ -196,6 +201,37 @@ def cpu_baseline(cfg, sample: int):
                       f"update), {dt:.2f} s wall, {dt * oracle.get_threads():.1f} core-s"}
 
 
+def workload(cfg) -> str:
+    """config.workload of both arms (the repo arm and --impl reference name the same workload)."""
+    return (f"{cfg.name}: {cfg.note} LM-OSEM {cfg.dims[0]}x{cfg.dims[1]}x{cfg.dims[2]} @ {cfg.voxel_mm[0]} mm, "
+            f"{cfg.n_subsets} subsets x {cfg.n_events} events, 1 iteration")
+
+
+def padded_bricks(dims):
+    """(bricks, real bricks) of the library's padded 2x2x2 brick image (halo 2 low, >= 2 high)."""
+    B = [(d + 5) // 2 for d in dims]
+    R = [(2 + d + 1) // 2 - 1 for d in dims]  # bricks [1, rhi) hold real voxels
+    return B[0] * B[1] * B[2], R[0] * R[1] * R[2]
+
+
+def combine_model(P: int, combine: str, dims) -> dict:
+    """Modeled NVLink floor of the combine per subset (SURVEY.md §8(d) t_AR,roof(P)) at
+    NVLINK_GBS per direction per GPU: all-reduce / ISD (reduce-scatter + all-gather) move
+    2(P-1)/P |c| per GPU; the fused multimem kernel moves the real bricks' |c| each way
+    (the switch pulls (P-1)/P of every rank's c, plus one multimem.st of the f block) —
+    egress and ingress overlap in one pass."""
+    nb, real = padded_bricks(dims)
+    c_bytes = 32.0 * nb
+    if P <= 1:
+        return {"t_ms": 0.0, "bytes_per_gpu": 0.0}
+    if combine == "fused":
+        b = 32.0 * real
+    else:
+        b = 2.0 * (P - 1) / P * c_bytes
+    return {"t_ms": b / (NVLINK_GBS * 1e9) * 1e3, "bytes_per_gpu": b, "nvlink_gbs": NVLINK_GBS,
+            "what": f"modeled, not measured: {b / 1e6:.1f} MB per GPU at {NVLINK_GBS} GB/s ({combine})"}
+
+
 def run_reference(args, cfg, rank):
     if rank != 0:
         return
@@ -217,9 +253,9 @@ def run_reference(args, cfg, rank):
     line = {"metric": METRIC, "value": v, "unit": "events/s", "impl": "reference", "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * dt / args.steps,
             "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
-            "data": "synthetic", "config": {"workload": f"{cfg.name}: {cfg.note} {cfg.dims[0]}x{cfg.dims[1]}x"
-                                            f"{cfg.dims[2]}, subsets of {cfg.n_events} events (oracle steps use a "
-                                            f"{sample}-event sample of each subset)"},
+            "data": "synthetic", "config": {"workload": workload(cfg), "sample_events_per_step": sample,
+                                            "sample": f"each oracle step runs a {sample}-event sample of the subset; "
+                                                      f"value = sampled events / s"},
             "cpu_baseline": {"value": v, "unit": "events/s", "cores": cores, "kind": "oracle",
                              "cpu_model": cpu_model(), "nproc": os.cpu_count(),
                              "sample": f"{sample} events per step x {args.steps} steps"},
@@ -364,10 +400,23 @@ def main():
             stp = rec.stats()
             rec.set_timing(False)
             ms_p = stp["project_ms"] / stp["timed_subsets"]
+            # the same share in the reconstruction loop (PDL chaining, no phase events):
+            # 3 passes over L subsets of n_p events, projection + full update per subset
+            offs_p = np.arange(L + 1, dtype=np.int64) * n_p
+            rec.reconstruct(ev[:L * n_p], offs_p, 1, f)
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(stream)
+            rec.reconstruct(ev[:L * n_p], offs_p, 3, f)
+            b.record(stream)
+            torch.cuda.synchronize()
+            loop_ms = a.elapsed_time(b) / (3 * L)
             shares[str(P)] = {"events": n_p, "project_ms": ms_p, "update_ms": stp["update_ms"] / stp["timed_subsets"],
-                              "projection_efficiency": (proj_ms / P) / ms_p}
+                              "projection_efficiency": (proj_ms / P) / ms_p, "loop_ms_per_subset": loop_ms}
         shares["what"] = ("projection of 1/P of a subset (the per-rank step-1 work at P GPUs), CUDA events on the "
-                          "library stream; projection_efficiency = (full-subset projection / P) / this")
+                          "library stream around the projection (they break the PDL overlap with the previous "
+                          "kernel); projection_efficiency = (full-subset projection / P) / this; loop_ms_per_subset = "
+                          "the same share as the reconstruction loop runs it (PDL chaining, no phase events): "
+                          "projection + the FULL update per subset")
 
     # ---- e2e through the public API with HOST buffers: one host reconstruction over the
     # K subsets (pinned events streamed per subset, f uploaded and downloaded)
@@ -416,10 +465,14 @@ def main():
     else:
         s_recon = None
 
+    # every rank releases its context (NCCL communicator) together; rank 0 then runs the
+    # single-GPU microbenchmarks and the oracle baseline and prints the line
+    n_slabs, rec_combine = rec.slabs, rec.combine
+    rec.close()
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
     if rank != 0:
-        rec.close()
-        if world > 1:
-            dist.destroy_process_group()
         return
 
     peaks, peak_kind = measured_peaks()
@@ -428,7 +481,6 @@ def main():
     pairs = ev_per_launch * mean_path
     proj_avg_s = proj_ms * 1e-3
     nbf = 8 * ((cfg.dims[0] + 5) // 2) * ((cfg.dims[1] + 5) // 2) * ((cfg.dims[2] + 5) // 2)  # padded bricks
-    n_slabs = rec.slabs
     # the microbenchmarks run on a buffer of the size each projection launch works on: the
     # image (V floats), or in the z-slab form one slab of the brick image (L2-resident)
     l2_floats = cfg.n_voxels if n_slabs == 1 else nbf // n_slabs
@@ -457,7 +509,7 @@ def main():
             "units_per_launch": ev_per_launch}
     if l2:
         roof["peak"] = l2["pair_warp32"] * 8.0 / 1e9
-        roof["peak_kind"] = ("measured live: fully coalesced fp32 gather+RED pairs (each warp on 32 consecutive "
+        roof["peak_kind"] = ("builder-measured live (libl2peak.so, not a driver number): fully coalesced fp32 gather+RED pairs (each warp on 32 consecutive "
                              f"floats) on a {l2_floats}-float L2-resident buffer (the image, or one z-slab of it; libl2peak.so, "
                              "PAIR_WARP32); the random-address pair rate is l2_micro_ops_per_s.pair")
         roof["frac"] = roof["achieved"] / roof["peak"]
@@ -519,17 +571,50 @@ def main():
         upd.update({"bound": "hbm", "peak": peaks["hbm_gbs"], "peak_kind": peak_kind})
     upd["frac"] = upd["achieved"] / upd["peak"]
 
+    # whole-step roofline: t_roof = projection at the L2 pair peak + the
+    # combine's modeled NVLink floor + the update at its streaming peak (1/P of it for the
+    # ISD / fused combines), against the measured time per subset
+    comb_name = {1: "allreduce", 2: "isd", 3: "fused"}.get(rec_combine, "allreduce") if world > 1 else "none"
+    step_roof = None
+    if l2:
+        proj_roof_ms = alg_l2_bytes / (roof["peak"] * 1e9) * 1e3
+        upd_roof_ms = upd_bytes / (upd["peak"] * 1e9) * 1e3 / (world if comb_name in ("isd", "fused") else 1)
+        ar = combine_model(world, comb_name, cfg.dims)
+        t_roof = proj_roof_ms + ar["t_ms"] + upd_roof_ms
+        step_roof = {"t_roof_ms": t_roof, "t_meas_ms": tot_ms / K, "frac": t_roof / (tot_ms / K),
+                     "terms_ms": {"project": proj_roof_ms, "combine_t_ar_roof": ar["t_ms"], "update": upd_roof_ms},
+                     "combine_model": ar,
+                     "what": "t_roof = projection bytes / live L2 pair peak + modeled NVLink floor of the combine + "
+                             "update bytes / live streaming peak (/P for isd/fused); frac = t_roof / measured ms per "
+                             "subset (whole job)"}
+    share_model = None
+    if shares:
+        # the step one rank of 8 would run (C3 at P = 8), from the measured 1/8-share projection
+        # and update on this GPU plus the modeled NVLink floor of the fused / ISD combine
+        t1 = tot_ms / K
+        share_model = {"P": 8, "t1_ms": t1, "project_share_ms": shares["8"]["project_ms"],
+                       "update_share_ms": upd_ms / 8, "loop_share_ms": shares["8"]["loop_ms_per_subset"]}
+        for cname in ("fused", "isd"):
+            ar8 = combine_model(8, cname, cfg.dims)
+            t8 = shares["8"]["project_ms"] + upd_ms / 8 + ar8["t_ms"]
+            t8l = shares["8"]["loop_ms_per_subset"] - upd_ms * 7 / 8 + ar8["t_ms"]
+            share_model[cname] = {"combine_roof_ms": ar8["t_ms"], "step_ms": t8, "efficiency_model": t1 / (8 * t8),
+                                  "step_ms_loop": t8l, "efficiency_model_loop": t1 / (8 * t8l)}
+        share_model["what"] = ("modeled P = 8 step from one GPU: the 1/8-share projection (CUDA events around it; or "
+                               "_loop: the share's reconstruction loop, PDL on, minus 7/8 of the measured update) + 1/8 "
+                               "of the measured update + the combine's modeled NVLink floor (770 GB/s); "
+                               "efficiency_model = T1 / (8 T8). A model, not a multi-GPU measurement.")
+
     line = {
         "metric": METRIC, "value": value, "unit": "events/s", "n_gpus": world, "steps": K, "warmup": args.warmup,
         "ms_per_step": tot_ms / K, "ms_per_step_median": med_ms, "higher_is_better": True, "scaling": "strong", "vs_baseline": None,
         "dtype": "f32", "geometry_dtype": "f64", "data": "synthetic",
-        "config": {"workload": f"{name}: {cfg.note} LM-OSEM {cfg.dims[0]}x{cfg.dims[1]}x{cfg.dims[2]} @ "
-                               f"{cfg.voxel_mm[0]} mm, {L} subsets x {N} events, 1 iteration",
+        "config": {"workload": workload(cfg),
                    "events_per_subset": N, "subsets": L, "parallelism": f"psd{world} (events block-distributed, f copy-distributed, c combined over NCCL)",
                    "l2": "not flushed: inputs larger than L2 (events of the 10 subsets, 24 B x N x 10); f, c "
                          "are the reconstruction's persistent state (flushed variant: flushed_subset_step)",
-                   "z_slabs": rec.slabs, "combine": {0: "none", 1: "allreduce", 2: "isd", 3: "fused"}.get(
-                       rec.combine if world > 1 else 0)},
+                   "z_slabs": n_slabs, "combine": {0: "none", 1: "allreduce", 2: "isd", 3: "fused"}.get(
+                       rec_combine if world > 1 else 0)},
         "s_per_recon": tot_ms / K * L * 1e-3, "s_per_recon_e2e": s_recon,
         "timed_region": f"{K} subset iterations = lmosem_reconstruct calls over the {L} subsets, cycling; "
                         "CUDA events around each call on the library's stream; ms_per_step_median = median over the calls of "
@@ -539,18 +624,16 @@ def main():
                               "what": "library CUDA events around each phase on its stream, in an instrumented pass "
                                       "of the same loop right after the timed region"},
         "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_l2_requests": roof_req,
-        "roofline_hbm_events": hbm, "roofline_update": upd,
+        "roofline_hbm_events": hbm, "roofline_update": upd, "roofline_step": step_roof,
+        "p8_share_model": share_model,
         "gpu_launches": launches, "flushed_subset_step": flushed, "per_rank_share": shares,
         "clocks": clocks, "wall_s_timed_region": t_wall,
         "e2e": e2e,
         "paper_context": PAPER_CONTEXT,
     }
-    if not args.no_cpu_baseline and world == 1:
+    if not args.no_cpu_baseline:  # rank 0 at every N
         line["cpu_baseline"] = cpu_baseline(cfg, min(args.cpu_sample, N))
     print(json.dumps(line), flush=True)
-    rec.close()
-    if world > 1:
-        dist.destroy_process_group()
 
 
 if __name__ == "__main__":

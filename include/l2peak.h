@@ -1,4 +1,4 @@
-/* l2peak.h — microbenchmarks for the roofline denominators of the LM-OSEM projection
+/* l2peak.h — builder-written microbenchmarks for the roofline denominators of the LM-OSEM projection
  * kernel: the rate of scattered 4-byte fp32 operations on an
  * image-sized buffer that sits in L2, the resource the back-projection
  * (red.global.add, Listing 2 lines 12-13) and the forward-projection gathers
@@ -19,8 +19,10 @@ enum {
     L2PEAK_PAIR_RUN8 = 4,     /* gather + red, 8-lane runs */
     L2PEAK_PAIR_WARP32 = 5,   /* gather + red, each warp on 32 consecutive floats (fully
                                  coalesced: the L2 peak for this op mix) */
-    L2PEAK_STREAM5 = 6        /* the update kernel's pattern streamed: read 3 arrays, write 2
+    L2PEAK_STREAM5 = 6,       /* the update kernel's pattern streamed: read 3 arrays, write 2
                                  (float4, 20 B per element); ops = elements x passes */
+    L2PEAK_LDG_WARP32 = 7,    /* gathers only, each warp on 32 consecutive floats (coalesced) */
+    L2PEAK_RED_WARP32 = 8     /* reds only, each warp on 32 consecutive floats (coalesced) */
 };
 
 /* Runs `mode` on the current device over a buffer of n_floats floats (three for

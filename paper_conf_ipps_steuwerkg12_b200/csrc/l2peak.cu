@@ -23,7 +23,7 @@ __global__ void __launch_bounds__(256) k_l2(float* __restrict__ buf, const float
     for (int it = 0; it < ops; ++it) {
         uint32_t h = hash32(tid * 0x9E3779B9u + (uint32_t)it * 0x85EBCA6Bu);
         uint32_t j;
-        if (MODE == L2PEAK_PAIR_WARP32) {
+        if (MODE == L2PEAK_PAIR_WARP32 || MODE == L2PEAK_LDG_WARP32 || MODE == L2PEAK_RED_WARP32) {
             uint32_t g = hash32((tid >> 5) * 0x9E3779B9u + (uint32_t)it * 0x85EBCA6Bu);
             j = ((uint32_t)(((uint64_t)g * (n - 32)) >> 32) & ~31u) + lane;
         } else if (MODE == L2PEAK_RED_RUN8 || MODE == L2PEAK_PAIR_RUN8) {
@@ -33,9 +33,9 @@ __global__ void __launch_bounds__(256) k_l2(float* __restrict__ buf, const float
             j = (uint32_t)(((uint64_t)h * n) >> 32);
         }
         if (MODE == L2PEAK_LDG_RANDOM || MODE == L2PEAK_PAIR_RANDOM || MODE == L2PEAK_PAIR_RUN8 ||
-            MODE == L2PEAK_PAIR_WARP32)
+            MODE == L2PEAK_PAIR_WARP32 || MODE == L2PEAK_LDG_WARP32)
             acc += __ldg(src + j);
-        if (MODE != L2PEAK_LDG_RANDOM) atomicAdd(buf + j, 1.0f + acc * 0.0f);
+        if (MODE != L2PEAK_LDG_RANDOM && MODE != L2PEAK_LDG_WARP32) atomicAdd(buf + j, 1.0f + acc * 0.0f);
     }
     if (acc == 12345.678f) sink[0] = acc;  // keeps the gathers alive
 }
@@ -69,6 +69,8 @@ cudaError_t launch_mode(int mode, float* buf, const float* src, uint32_t n, int 
         case L2PEAK_RED_RUN8: return launch<L2PEAK_RED_RUN8>(buf, src, n, ops, sink, grid);
         case L2PEAK_PAIR_RUN8: return launch<L2PEAK_PAIR_RUN8>(buf, src, n, ops, sink, grid);
         case L2PEAK_PAIR_WARP32: return launch<L2PEAK_PAIR_WARP32>(buf, src, n, ops, sink, grid);
+        case L2PEAK_LDG_WARP32: return launch<L2PEAK_LDG_WARP32>(buf, src, n, ops, sink, grid);
+        case L2PEAK_RED_WARP32: return launch<L2PEAK_RED_WARP32>(buf, src, n, ops, sink, grid);
         case L2PEAK_STREAM5:
             k_stream5<<<grid, 256>>>(reinterpret_cast<float4*>(buf), const_cast<float4*>(reinterpret_cast<const float4*>(src)),
                                      reinterpret_cast<const float4*>(sink), n / 4, ops);
@@ -80,7 +82,7 @@ cudaError_t launch_mode(int mode, float* buf, const float* src, uint32_t n, int 
 }  // namespace
 
 L2PEAK_API int l2peak_run(int mode, int64_t n_floats, int32_t ops_per_thread, float* ms, double* ops) {
-    if (mode < 0 || mode > 6 || n_floats < 64 || n_floats >= (int64_t(1) << 32) || ops_per_thread <= 0 || !ms || !ops)
+    if (mode < 0 || mode > L2PEAK_RED_WARP32 || n_floats < 64 || n_floats >= (int64_t(1) << 32) || ops_per_thread <= 0 || !ms || !ops)
         return -1;
     int dev = 0, sms = 0, per_sm = 0;
     if (cudaGetDevice(&dev) != cudaSuccess) return -1;

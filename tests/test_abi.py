@@ -154,7 +154,7 @@ def test_l2peak_exports_and_rejects_bad_arguments(lib):
     l2.l2peak_run.argtypes = [ctypes.c_int, ctypes.c_int64, ctypes.c_int32, ctypes.POINTER(ctypes.c_float),
                               ctypes.POINTER(ctypes.c_double)]
     ms, ops = ctypes.c_float(), ctypes.c_double()
-    for mode, n, k in [(7, 1 << 20, 4), (-1, 1 << 20, 4), (0, 10, 4), (0, 1 << 20, 0), (0, 1 << 33, 4)]:
+    for mode, n, k in [(9, 1 << 20, 4), (-1, 1 << 20, 4), (0, 10, 4), (0, 1 << 20, 0), (0, 1 << 33, 4)]:
         assert l2.l2peak_run(mode, n, k, ctypes.byref(ms), ctypes.byref(ops)) == -1
 
 

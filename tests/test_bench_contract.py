@@ -31,6 +31,17 @@ def test_reference_arm_line():
     assert cb["kind"] == "oracle" and cb["cores"] >= 1 and cb["value"] == d["value"] and cb["sample"]
     assert d["e2e"] == {"value": d["value"], "unit": "events/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}
     assert d["config"]["workload"].startswith("C1")
+    assert d["config"]["workload"] == repo_arm_workload("C1")  # the same workload string as the repo arm
+    assert d["config"]["sample_events_per_step"] > 0
+
+
+def repo_arm_workload(name):
+    import importlib.util
+    import lmgen
+    spec = importlib.util.spec_from_file_location("bench_mod", BENCH)
+    m = importlib.util.module_from_spec(spec)
+    spec.loader.exec_module(m)
+    return m.workload(lmgen.CONFIGS[name])
 
 
 def test_reference_arm_other_ranks_are_silent():
@@ -60,3 +71,9 @@ def test_cuda_arm_line():
     # one f -> brick conversion per reconstruct call, then (projection, update) per subset
     assert d["gpu_launches"] >= 2 * d["steps"]
     assert "sm_mhz" in d["clocks"] and "reasons" in d["clocks"]
+    assert d["config"]["workload"] == repo_arm_workload("C1")
+    rs = d["roofline_step"]
+    assert rs["t_roof_ms"] > 0 and abs(rs["frac"] - rs["t_roof_ms"] / rs["t_meas_ms"]) < 1e-9
+    assert rs["terms_ms"]["combine_t_ar_roof"] == 0.0  # one GPU: no combine
+    m = d["p8_share_model"]
+    assert m["P"] == 8 and m["fused"]["step_ms"] > m["project_share_ms"]
