@@ -88,7 +88,8 @@ struct lmosem_ctx {
     float* norm = nullptr;     // s in bricks (halo = 0)
     float* scratch = nullptr;  // V floats, row layout (norm upload)
     int cap = 0;               // path-piece capacity per warp of the full clip box (the largest launch)
-    int slabs_forced = 0;      // z-slab count (0 = automatic from the L2 budget)
+    int slabs_forced = 0;      // slab count (0 = automatic from the L2 budget)
+    int slab_axis = 2;         // slabs along z, or along the one axis longer than kMaxBox
     float* fp_acc = nullptr;   // per-event forward projections of the z-slab passes
     unsigned long long* work = nullptr;  // k_project work counters (one per launch in a step)
     int work_next = 0;
@@ -474,16 +475,36 @@ lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
     return LMOSEM_OK;
 }
 
-// Number of z-slabs for the projection: the brick image slab of a pass should stay
-// L2-resident (L2 126 MB; a 72 MB budget per image slab leaves room for the event stream
-// and the per-event fp array; measured at C4, 208 MB: 2/3/4/5 slabs 27.1/24.5/25.2/26.3
-// ms). 1 = the single fused pass.
+// Largest clip-box extent (voxels) whose per-warp path buffer (3 pieces per dominant-axis
+// slab, 8 B each, 8 warps per CTA) fits the 227 KB of opt-in shared memory of sm_100a.
+constexpr int kMaxBox = 1210;
+
+// Largest slab extent along `axis` when it is cut into K even-aligned slabs (slab_geom).
+int max_slab_extent(int n_axis, int K) {
+    const int half = n_axis / 2;
+    int m = 0;
+    for (int k = 0; k < K; ++k) {
+        const int lo = 2 * (int)((int64_t)half * k / K);
+        const int hi = (k == K - 1) ? n_axis : 2 * (int)((int64_t)half * (k + 1) / K);
+        m = std::max(m, hi - lo);
+    }
+    return m;
+}
+
+// Number of slabs for the projection, along ctx->slab_axis (z, or the one axis longer than
+// kMaxBox): the brick image slab of a pass should stay L2-resident (L2 126 MB; a 72 MB
+// budget per image slab leaves room for the event stream and the per-event fp array;
+// measured at C4, 208 MB: 2/3/4/5 slabs 27.1/24.5/25.2/26.3 ms), and no slab may be longer
+// than kMaxBox along its axis (the path buffer). 1 = the single fused pass.
 int n_slabs(const lmosem_ctx* ctx) {
-    const int max_slabs = std::max(1, ctx->dims[2] / 2);
-    if (ctx->slabs_forced > 0) return std::min(ctx->slabs_forced, max_slabs);
+    const int n_axis = ctx->dims[ctx->slab_axis];
+    const int max_slabs = std::max(1, n_axis / 2);
+    int k_min = 1;  // the path-buffer bound (> 1 only for an axis longer than kMaxBox)
+    while (k_min < max_slabs && max_slab_extent(n_axis, k_min) > kMaxBox) ++k_min;
+    if (ctx->slabs_forced > 0) return std::max(k_min, std::min(ctx->slabs_forced, max_slabs));
     const double bytes = 4.0 * (double)ctx->nbf;
     const double budget = 72.0 * 1024 * 1024;
-    return std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget)));
+    return std::max(k_min, std::min(max_slabs, std::max(1, (int)std::ceil(bytes / budget))));
 }
 
 #ifndef LMOSEM_STATIC_BATCH
@@ -582,10 +603,11 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
 }
 
 lmk::GridGeom slab_geom(const lmosem_ctx* ctx, int k, int K) {
-    const int half = ctx->dims[2] / 2;  // slab boundaries on even z (brick aligned)
+    const int a = ctx->slab_axis;
+    const int half = ctx->dims[a] / 2;  // slab boundaries on even coordinates (brick aligned)
     lmk::GridGeom g = ctx->geom;
-    g.clo[2] = 2 * (int)((int64_t)half * k / K);
-    g.chi[2] = (k == K - 1) ? ctx->dims[2] : 2 * (int)((int64_t)half * (k + 1) / K);
+    g.clo[a] = 2 * (int)((int64_t)half * k / K);
+    g.chi[a] = (k == K - 1) ? ctx->dims[a] : 2 * (int)((int64_t)half * (k + 1) / K);
     return g;
 }
 
@@ -1002,8 +1024,9 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     }
     if (V >= (int64_t(1) << 31)) return LMOSEM_EINVAL;
     // per-warp path buffer: 8 warps x 3 pieces per slab x 8 B must fit the 227 KB opt-in
-    // shared memory of sm_100a (checked again against the device below)
-    if (std::max(dims[0], std::max(dims[1], dims[2])) > 1210) return LMOSEM_EINVAL;
+    // shared memory of sm_100a for every clip box: one axis longer than kMaxBox is cut into
+    // slabs (n_slabs), two are not supported (checked again against the device below)
+    if ((dims[0] > kMaxBox) + (dims[1] > kMaxBox) + (dims[2] > kMaxBox) > 1) return LMOSEM_EINVAL;
     int rank = 0, world = 1;
     if (dist) {
         rank = dist->rank;
@@ -1062,8 +1085,12 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
             ctx->geom.B[k] = (int)(m[k] - M[k] / 2);
         }
     }
-    // whole-volume path buffer (the largest launch; see path_cap)
-    ctx->cap = path_cap(std::max(dims[0], std::max(dims[1], dims[2])));
+    // slabs along z, or along the one axis longer than kMaxBox
+    ctx->slab_axis = 2;
+    for (int k = 0; k < 3; ++k)
+        if (dims[k] > kMaxBox) ctx->slab_axis = k;
+    // path buffer of the largest clip box (the whole volume, or a slab of it; see path_cap)
+    ctx->cap = path_cap(std::min(kMaxBox, std::max(dims[0], std::max(dims[1], dims[2]))));
     ctx->proj_smem = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
 
     lmosem_status s = LMOSEM_OK;

@@ -92,7 +92,7 @@ def _init(lib, dims, vox, norm_ptr=1, dist=None):
 @pytest.mark.parametrize("dims,vox", [((0, 4, 4), (1, 1, 1)), ((4, -1, 4), (1, 1, 1)),
                                       ((4, 4, 4), (0, 1, 1)), ((4, 4, 4), (1, float("nan"), 1)),
                                       ((4, 4, 4), (1, 1, float("inf"))), ((2048, 2048, 1024), (1, 1, 1)),
-                                      ((4, 4, 1211), (1, 1, 1)), ((1211, 2, 2), (1, 1, 1))])
+                                      ((4, 1211, 1211), (1, 1, 1)), ((1300, 2, 1300), (1, 1, 1))])
 def test_init_einval_before_cuda(lib, dims, vox):
     st, h = _init(lib, dims, vox)
     assert st == L.EINVAL and not h.value
