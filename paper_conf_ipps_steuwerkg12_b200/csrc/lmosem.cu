@@ -535,13 +535,25 @@ constexpr int kWorkSlots = 64;
 // warp's buffer starts 32-byte aligned (the tile is staged with 16-byte vector stores).
 int path_cap(int m) { return (std::max(96, 3 * m) + 3) & ~3; }
 
+#ifndef LMOSEM_CAP_SUM
+#define LMOSEM_CAP_SUM 1  // 0: size path buffers by 3 pieces per slab only (A/B)
+#endif
+
 // Path-buffer entries per warp for one launch: the forward-only modes (1, 2) keep no path
-// and need only the 32-event tile (96 entries); the others hold <= 3 pieces per dominant-axis
-// slab of the launch's clip box (a z-slab pass: max(nx, ny, slab height)).
+// and need only the 32-event tile (96 entries); the others hold the pieces of one LOR in the
+// launch's clip box of extents e0, e1, e2 (the volume, or a slab of it). Two bounds: <= 3
+// pieces per dominant-axis slab (3 max e), and one piece per slab plus one per minor-axis
+// plane crossing: the minor positions stay inside the box up to rounding (lor_setup's guard),
+// so each minor axis crosses at most e + 2 planes -> e_a + (e_b + 2) + (e_c + 2) <= sum e + 4.
+// The smaller bound (C2: 584 instead of 840 pieces) leaves the SM more L1 for the gathers.
 int launch_cap(int mode, const lmk::GridGeom& g) {
     if (mode == 1 || mode == 2) return 96;
-    int m = 0;
-    for (int k = 0; k < 3; ++k) m = std::max(m, g.chi[k] - g.clo[k]);
+    int m = 0, sum = 0;
+    for (int k = 0; k < 3; ++k) {
+        m = std::max(m, g.chi[k] - g.clo[k]);
+        sum += g.chi[k] - g.clo[k];
+    }
+    if (LMOSEM_CAP_SUM && sum + 4 < 3 * m) return (std::max(96, sum + 4) + 3) & ~3;
     return path_cap(m);
 }
 
