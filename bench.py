@@ -490,7 +490,7 @@ def main():
     alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)
     traffic, sectors = None, None
     try:
-        with open(os.path.join(ROOT, "profiles", "r01_traffic.json")) as fh:
+        with open(os.path.join(ROOT, "profiles", "r02_traffic.json")) as fh:
             tr = json.load(fh).get(name)
         if tr and tr.get("launches_per_step", 1) == (2 * n_slabs if n_slabs > 1 else 1):
             traffic = tr["dram_bytes_read_per_launch"] + tr["dram_bytes_write_per_launch"]
@@ -503,7 +503,7 @@ def main():
     roof = {"kernel": kname, "bound": "l2",
             "achieved": alg_l2_bytes / proj_avg_s / 1e9, "unit": "GB/s", "traffic": traffic,
             "traffic_note": "DRAM bytes per launch, summed over one subset's launches in the z-slab form (ncu --set "
-                            "full, profiles/r01_traffic.json); the algorithmic bytes are L2 traffic (the images, or "
+                            "full, profiles/r02_traffic.json); the algorithmic bytes are L2 traffic (the images, or "
                             "the slab being projected, stay L2-resident)",
             "per_unit": f"{mean_path} path elements x (4 B f gather + 4 B c RED) + 24 B event per event",
             "units_per_launch": ev_per_launch}
@@ -535,7 +535,7 @@ def main():
         roof_sec = {"bound": "l2_sectors", "achieved": sectors / proj_avg_s, "peak": peak_sec, "unit": "sectors/s",
                     "frac": sectors / proj_avg_s / peak_sec, "sectors_per_launch": sectors,
                     "path_elements_per_sector": 2 * pairs / sectors,
-                    "what": "ncu L2 sectors of k_project (gathers + REDs, profiles/r01_traffic.json) / live duration, "
+                    "what": "ncu L2 sectors of k_project (gathers + REDs, profiles/r02_traffic.json) / live duration, "
                             "vs the max sector rate over the live L2 microbenchmark modes (random RED, random gather, "
                             "random / 8-lane / 32-lane gather+RED pairs)"}
     # request view (DESIGN.md §7 summary): the SM->L2 request interface takes about one request
@@ -550,7 +550,7 @@ def main():
         roof_req = {"bound": "l2_request_interface", "achieved": cyc / proj_avg_s, "peak": peak_req,
                     "unit": "request cycles/s", "frac": cyc / proj_avg_s / peak_req,
                     "request_cycles_per_launch": cyc, "ncu_req_cycles_active_pct": tr.get("req_cycles_active_pct"),
-                    "what": "(gather requests + RED sectors) per launch (ncu, profiles/r01_traffic.json; summed over "
+                    "what": "(gather requests + RED sectors) per launch (ncu, profiles/r02_traffic.json; summed over "
                             "a subset's launches in the z-slab form) / live duration, vs one request cycle per SM "
                             "clock (SMs x median SM clock under load)"}
     hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)) / proj_avg_s / 1e9,

@@ -4,6 +4,10 @@ exchange step costs on the device apart from NVLink traffic — kernel launches,
 own copies, the fused kernel's barriers and re-zeroing — next to the plain update
 (diagnostic)."""
 import json
+import os
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 
 import numpy as np
 import torch

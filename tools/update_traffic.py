@@ -1,5 +1,5 @@
 #!/usr/bin/env python
-"""Writes one config's entry of profiles/r01_traffic.json (read by bench.py) from an ncu
+"""Writes one config's entry of profiles/r02_traffic.json (read by bench.py) from an ncu
 --set full capture of that config's projection: DRAM bytes and L2 sectors (gathers, REDs)
 per launch of the fused kernel, or summed over the launches of one subset step (the C4
 z-slab form: 3 pass-A + 3 pass-B launches).
@@ -12,7 +12,7 @@ import subprocess
 import sys
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
-PATH = os.path.join(ROOT, "profiles", "r01_traffic.json")
+PATH = os.environ.get("LMOSEM_TRAFFIC_JSON") or os.path.join(ROOT, "profiles", "r02_traffic.json")
 
 
 def main(rep, summary, config="C2", per_step=1):
