@@ -158,3 +158,54 @@ def test_fuzz_scaled_and_short(pkg, seed, scale):
     got = f.cpu().numpy().astype(np.float64)
     mm = ref > 1e-3 * ref.max()
     assert float(np.max(np.abs(got[mm] - ref[mm]) / ref[mm])) <= 1e-4
+
+
+@pytest.mark.parametrize("seed", range(SEED0, SEED0 + max(1, (16 * N_CASES) // 64)))
+def test_fuzz_loopback_world(pkg, seed):
+    """Random emulated worlds (P = 1..8 ranks of the loopback transport on this GPU, one host
+    thread each), random combine (ALLREDUCE / ISD / FUSED), random volume, voxel sizes,
+    slab count and subset offsets (empty subsets included): a reconstruction through
+    lmosem_reconstruct on every rank against the oracle's, with bitwise-equal replicas
+    (PAPER.md lines 476-485, 509-518)."""
+    import threading
+    dims, vox, ev, s, f0, slabs = case(400 + seed)
+    rng = np.random.default_rng(500 + seed)
+    P = int(rng.integers(1, 9))
+    combine = int(rng.integers(1, 4))
+    L = int(rng.integers(1, 5))
+    off = np.concatenate([[0], np.sort(rng.integers(0, len(ev) + 1, L - 1)), [len(ev)]]).astype(np.int64)
+    g = oracle.geom(dims, vox)
+    ref = oracle.reconstruct(g, ev, off, 1, s, f0.astype(np.float64))
+    group = pkg.Loopback(P)
+    recs = [pkg.Reconstructor(dims, vox, dev(s), stream=torch.cuda.Stream(), loopback=(group, r)) for r in range(P)]
+    fs = []
+    for rec in recs:
+        rec.set_slabs(slabs)
+        rec.set_combine(combine)
+        fs.append(dev(f0))
+    d_ev = dev(ev)
+    torch.cuda.synchronize()
+    errs = []
+
+    def work(r):
+        try:
+            recs[r].reconstruct(d_ev, off, 1, fs[r])
+            recs[r].synchronize()
+        except Exception as e:  # noqa: BLE001
+            errs.append(e)
+    th = [threading.Thread(target=work, args=(r,)) for r in range(P)]
+    for t in th:
+        t.start()
+    for t in th:
+        t.join(timeout=300)
+    assert not errs, errs
+    out = [f.cpu().numpy() for f in fs]
+    for rec in recs:
+        rec.close()
+    group.close()
+    for r in range(1, P):
+        assert np.array_equal(out[r], out[0]), (P, combine, r)
+    got = out[0].astype(np.float64)
+    assert float(np.linalg.norm(got - ref) / np.linalg.norm(ref)) <= 1e-3, (P, combine, dims, slabs)
+    mm = ref > 1e-3 * ref.max()
+    assert float(np.max(np.abs(got[mm] - ref[mm]) / ref[mm])) <= 1e-4 * (1 + L), (P, combine, dims, slabs)
