@@ -257,8 +257,9 @@ lmosem_status lmosem_update(lmosem_ctx* ctx, float* f, float* c);
 /* Waits for all work enqueued by this context. Reports asynchronous kernel faults. With an
  * NCCL communicator it is a watchdog: ncclCommGetAsyncError is polled, and after
  * LMOSEM_TIMEOUT_S seconds (default 300) without completion — a peer rank that died or never
- * reached the collective — the communicator is aborted and ENCCL returned (the context then
- * answers ESTATE). The synchronous host/file reconstructions wait the same way. */
+ * reached the collective — ENCCL is returned; the context then answers ESTATE and
+ * lmosem_destroy aborts its communicator (ncclCommAbort) before releasing it. The
+ * synchronous host/file reconstructions wait the same way. */
 lmosem_status lmosem_synchronize(lmosem_ctx* ctx);
 
 /* Enables (1) / disables (0) per-phase CUDA-event timing; enabling clears the times. */

@@ -43,6 +43,13 @@ struct PhaseMarks {
 #define LMOSEM_FUSED_CTAS_PER_SM 4  // fused combine: CTAs (and LSA barriers) per SM
 #endif
 
+#ifndef LMOSEM_WIDE_N
+// fused launches of >= this many events use the 28-warp shape (MODE 6). Measured on one
+// B200 (profiles/r02_shape_ab): C2 whole subset 0.964 -> 0.947 ms, 1/2 share 0.488 -> 0.487;
+// 1/4 and 1/8 shares slower (0.255 -> 0.259, 0.143 -> 0.149): fewer events per warp
+#define LMOSEM_WIDE_N 400000
+#endif
+
 // reconstruct_host pipelines the final f download in kPipe brick z-ranges
 constexpr int kPipe = 8;
 // the first subset's upload: kInChunks parts of growing size (1/16, 3/16, 4/16, 8/16 of the
@@ -90,6 +97,7 @@ struct lmosem_ctx {
     int cap = 0;               // path-piece capacity per warp of the full clip box (the largest launch)
     int slabs_forced = 0;      // slab count (0 = automatic from the L2 budget)
     int slab_axis = 2;         // slabs along z, or along the one axis longer than kMaxBox
+    int64_t wide_n = LMOSEM_WIDE_N;  // fused launches of at least this many events run MODE 6 (LMOSEM_WIDE_N)
     float* fp_acc = nullptr;   // per-event forward projections of the z-slab passes
     unsigned long long* work = nullptr;  // k_project work counters (one per launch in a step)
     int work_next = 0;
@@ -571,7 +579,8 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
         case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2>, lmk::proj_threads_of(2), smem)); break;
         case 3: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<3>, lmk::proj_threads_of(3), smem)); break;
         case 4: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<4>, lmk::proj_threads_of(4), smem)); break;
-        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<5>, lmk::proj_threads_of(5), smem)); break;
+        case 5: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<5>, lmk::proj_threads_of(5), smem)); break;
+        default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<6>, lmk::proj_threads_of(6), smem)); break;
     }
     b = std::max(1, b);
     ctx->occ.push_back({mode, smem, b});
@@ -608,7 +617,8 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
         case 2: k = lmk::k_project<2>; break;
         case 3: k = lmk::k_project<3>; break;
         case 4: k = lmk::k_project<4>; break;
-        default: k = lmk::k_project<5>; break;
+        case 5: k = lmk::k_project<5>; break;
+        default: k = lmk::k_project<6>; break;
     }
     CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch, gdiv));
     return LMOSEM_OK;
@@ -630,8 +640,11 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
     if (n <= 0) return LMOSEM_OK;
     const float* evf = reinterpret_cast<const float*>(ev);
     const int K = n_slabs(ctx);
-    if (mode == 1 || K == 1)  // the fused pass gathers through the texture pipe when it can (MODE 5)
-        return launch_mode(ctx, (mode == 0 && ctx->geom.tex_fb) ? 5 : mode, evf, n, fp_out, ctx->geom);
+    if (mode == 1 || K == 1) {  // the fused pass gathers through the texture pipe when it can (MODE 5)
+        int m = (mode == 0 && ctx->geom.tex_fb) ? 5 : mode;
+        if (m == 5 && n >= ctx->wide_n) m = 6;  // large launch: 28 warps per SM
+        return launch_mode(ctx, m, evf, n, fp_out, ctx->geom);
+    }
     lmosem_status s;
     if (mode == 4) {
         for (int k = 0; k < K; ++k)
@@ -676,8 +689,8 @@ struct Nvtx {
     ~Nvtx() { nvtxRangePop(); }
 };
 
-// After a failed or timed-out collective: abort the communicator so NCCL kernels stuck on
-// a dead peer exit, and forget every handle tied to it (the context is then failed).
+// Destroying a failed context: abort the communicator so NCCL kernels stuck on a dead peer
+// exit, and forget every handle tied to it.
 void abort_comm(lmosem_ctx* ctx) {
     if (!ctx->comm) return;
     if (ctx->abort_flag) *(volatile int*)ctx->abort_flag = 1;
@@ -688,10 +701,18 @@ void abort_comm(lmosem_ctx* ctx) {
     ctx->reg_c = ctx->reg_fb = nullptr;
 }
 
+// A collective failed or timed out: the context is failed (ENCCL, then ESTATE) and its
+// communicator is aborted by lmosem_destroy (ncclCommAbort takes ~1 s of NCCL teardown, so
+// the failing call returns first; the abort flag already stops the library's own kernels).
+lmosem_status comm_failure(lmosem_ctx* ctx, lmosem_status s, const std::string& msg) {
+    if (ctx->abort_flag) *(volatile int*)ctx->abort_flag = 1;
+    return fail(ctx, s, msg);
+}
+
 // Waits until `ev` (or, with ev == nullptr, stream `st`) completes. With an NCCL
 // communicator this is a watchdog: it polls ncclCommGetAsyncError and gives up after
-// LMOSEM_TIMEOUT_S seconds (a peer that died or never joined the collective), aborting the
-// communicator; the result is ENCCL and the context answers ESTATE from then on.
+// LMOSEM_TIMEOUT_S seconds (a peer that died or never joined the collective); the result is
+// ENCCL, the context answers ESTATE from then on and lmosem_destroy aborts the communicator.
 lmosem_status wait_done(lmosem_ctx* ctx, cudaStream_t st, cudaEvent_t ev = nullptr) {
     if (!ctx->comm) {
         CK(ev ? cudaEventSynchronize(ev) : cudaStreamSynchronize(st));
@@ -702,24 +723,20 @@ lmosem_status wait_done(lmosem_ctx* ctx, cudaStream_t st, cudaEvent_t ev = nullp
     for (;;) {
         const cudaError_t e = ev ? cudaEventQuery(ev) : cudaStreamQuery(st);
         if (e == cudaSuccess) return LMOSEM_OK;
-        if (e != cudaErrorNotReady) {
-            abort_comm(ctx);
-            return fail(ctx, LMOSEM_ECUDA, std::string("wait: ") + cudaGetErrorString(e));
-        }
+        if (e != cudaErrorNotReady)
+            return comm_failure(ctx, LMOSEM_ECUDA, std::string("wait: ") + cudaGetErrorString(e));
         ncclResult_t ae = ncclSuccess;
         const ncclResult_t r = ncclCommGetAsyncError(ctx->comm, &ae);
-        if (r != ncclSuccess || (ae != ncclSuccess && ae != ncclInProgress)) {
-            const std::string why = ncclGetErrorString(r != ncclSuccess ? r : ae);
-            abort_comm(ctx);
-            return fail(ctx, LMOSEM_ENCCL, "nccl async error: " + why + " (communicator aborted)");
-        }
+        if (r != ncclSuccess || (ae != ncclSuccess && ae != ncclInProgress))
+            return comm_failure(ctx, LMOSEM_ENCCL,
+                                std::string("nccl async error: ") + ncclGetErrorString(r != ncclSuccess ? r : ae) +
+                                    " (the communicator is aborted by lmosem_destroy)");
         const double waited = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
-        if (waited > limit) {
-            abort_comm(ctx);
-            return fail(ctx, LMOSEM_ENCCL, "timed out after " + std::to_string((int)limit) +
-                                               " s (LMOSEM_TIMEOUT_S) waiting for the stream: a peer rank stalled "
-                                               "or died; communicator aborted");
-        }
+        if (waited > limit)
+            return comm_failure(ctx, LMOSEM_ENCCL,
+                                "timed out after " + std::to_string((int)limit) +
+                                    " s (LMOSEM_TIMEOUT_S) waiting for the stream: a peer rank stalled or died; the "
+                                    "communicator is aborted by lmosem_destroy");
         std::this_thread::sleep_for(std::chrono::microseconds(50));
     }
 }
@@ -1118,6 +1135,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (!cuda(cudaGetDeviceProperties(&prop, ctx->device), "cudaGetDeviceProperties")) return bail(s);
     ctx->num_sms = prop.multiProcessorCount;
     if (const char* e = std::getenv("LMOSEM_PDL")) ctx->pdl = e[0] != '0';  // A/B switch (default on)
+    if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {
         if (!cuda(cudaHostAlloc(&ctx->abort_flag, sizeof(int), cudaHostAllocMapped), "cudaHostAlloc(abort flag)"))
@@ -1141,6 +1159,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
         cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
         cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
         cuda(cudaFuncSetAttribute(lmk::k_project<5>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<6>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
     }
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
@@ -1632,10 +1651,8 @@ LMOSEM_API lmosem_status lmosem_synchronize(lmosem_ctx* ctx) {
     if (ctx->comm) {
         ncclResult_t async_err = ncclSuccess;
         NK(ncclCommGetAsyncError(ctx->comm, &async_err));
-        if (async_err != ncclSuccess) {
-            abort_comm(ctx);
-            return fail(ctx, LMOSEM_ENCCL, std::string("nccl async: ") + ncclGetErrorString(async_err));
-        }
+        if (async_err != ncclSuccess)
+            return comm_failure(ctx, LMOSEM_ENCCL, std::string("nccl async: ") + ncclGetErrorString(async_err));
     }
     return LMOSEM_OK;
 }
@@ -1663,6 +1680,9 @@ LMOSEM_API lmosem_status lmosem_get_stats(lmosem_ctx* ctx, lmosem_stats* out) {
 
 LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (!ctx) return LMOSEM_OK;
+    // a failed context may have a collective stuck on a dead peer: abort the communicator
+    // before waiting for the streams (its kernels then exit)
+    if (ctx->failed) abort_comm(ctx);
     if (ctx->stream) cudaStreamSynchronize(ctx->stream);
     if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
     if (ctx->comm) {

@@ -364,6 +364,12 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #ifndef LMK_MIN_BLOCKS
 #define LMK_MIN_BLOCKS 3     // CTAs per SM
 #endif
+#ifndef LMK_WIDE_CTA_THREADS
+#define LMK_WIDE_CTA_THREADS 224  // CTA size of MODE 6 (the fused pass of large launches)
+#endif
+#ifndef LMK_WIDE_MIN_BLOCKS
+#define LMK_WIDE_MIN_BLOCKS 4
+#endif
 #ifndef LMK_SLAB_CTA_THREADS
 #define LMK_SLAB_CTA_THREADS 128  // CTA size of the z-slab passes (modes 2, 3)
 #endif
@@ -401,11 +407,15 @@ __device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.lau
 __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
 
 template <int MODE>
-constexpr int proj_min_blocks() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN_BLOCKS : LMK_MIN_BLOCKS; }
+constexpr int proj_min_blocks() {
+    return (MODE == 2 || MODE == 3) ? LMK_SLAB_MIN_BLOCKS : (MODE == 6 ? LMK_WIDE_MIN_BLOCKS : LMK_MIN_BLOCKS);
+}
 template <int MODE>
-constexpr int proj_threads() { return (MODE == 2 || MODE == 3) ? LMK_SLAB_CTA_THREADS : LMK_CTA_THREADS; }
+constexpr int proj_threads() {
+    return (MODE == 2 || MODE == 3) ? LMK_SLAB_CTA_THREADS : (MODE == 6 ? LMK_WIDE_CTA_THREADS : LMK_CTA_THREADS);
+}
 __host__ __device__ constexpr int proj_threads_of(int mode) {
-    return (mode == 2 || mode == 3) ? LMK_SLAB_CTA_THREADS : LMK_CTA_THREADS;
+    return (mode == 2 || mode == 3) ? LMK_SLAB_CTA_THREADS : (mode == 6 ? LMK_WIDE_CTA_THREADS : LMK_CTA_THREADS);
 }
 
 // Dynamic shared memory: per warp `cap` path pieces (int j, float len) packed as int2
@@ -420,6 +430,9 @@ __host__ __device__ constexpr int proj_threads_of(int mode) {
 //         projection).
 // MODE 5: MODE 0 with the gathers of f through the texture pipe (tex1Dfetch on g.tex_fb),
 //         the default for the fused pass when the brick f fits a 1-D linear texture.
+// MODE 6: MODE 5 with 28 warps per SM (224 threads x 4 CTAs) instead of 24: large launches
+//         (a whole C2 subset: -1.7 %); a rank's small share keeps MODE 5 (fewer, larger
+//         claims per warp).
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
 template <int MODE>
@@ -428,9 +441,9 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                                                              float* __restrict__ fp, GridGeom g, int cap,
                                                              unsigned long long* __restrict__ work, int batch,
                                                              int gdiv) {
-    constexpr bool kGather = MODE <= 2 || MODE == 5;  // forward projection in this launch
-    constexpr bool kScatter = MODE == 0 || MODE == 3 || MODE == 4 || MODE == 5;  // back-projection
-    constexpr bool kTex = MODE == 5;  // gathers of f through the texture path
+    constexpr bool kGather = MODE <= 2 || MODE >= 5;  // forward projection in this launch
+    constexpr bool kScatter = MODE == 0 || MODE >= 3;  // back-projection
+    constexpr bool kTex = MODE >= 5;  // gathers of f through the texture path
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;

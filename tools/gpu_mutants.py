@@ -58,8 +58,8 @@ MUTANTS = [
      "2 * bx + ((q >> 1) & 1), 2 * by + (q & 1)", True),
     ("PDL: no wait before the first image access", K, "            pdl_wait();\n            dep_ready = true;",
      "            dep_ready = true;", False),
-    ("z-slab boundaries off by one brick", H, "g.clo[2] = 2 * (int)((int64_t)half * k / K);",
-     "g.clo[2] = 2 * (int)((int64_t)half * k / K) + (k > 0 ? 2 : 0);", False),
+    ("z-slab boundaries off by one brick", H, "g.clo[a] = 2 * (int)((int64_t)half * k / K);",
+     "g.clo[a] = 2 * (int)((int64_t)half * k / K) + (k > 0 ? 2 : 0);", False),
     # the multi-rank combine (round 2: caught by tests/test_loopback_gpu.py, P ranks on one GPU)
     ("combine: events not block-split (every rank projects the whole subset)", H,
      "if (whole_subset) block_range(n, ctx->rank, ctx->world, &b, &e);", "if (false) block_range(n, ctx->rank, ctx->world, &b, &e);", False),
