@@ -302,6 +302,23 @@ class Reconstructor:
         self._check(self._lib.lmosem_reconstruct(self._h, ep, off.ctypes.data, off.size - 1, int(n_iterations),
                                                  _dev_ptr(f, "float32", self.V)))
 
+    def resume(self, events, offsets, n_iterations, f, start_iteration: int, start_subset: int):
+        """Checkpoint / resume: continue a reconstruction of n_iterations passes
+        from a checkpoint taken after subset start_subset - 1 of iteration start_iteration
+        (f = the checkpointed image, e.g. copied out after a reconstruct call that stopped
+        there): the rest of that iteration, then the remaining full iterations — the same
+        sequence of subset iterations as one uninterrupted lmosem_reconstruct call (two calls
+        of the C ABI; nothing is computed here)."""
+        off = self._offsets(offsets, self._events_ptr(events)[1])
+        L = off.size - 1
+        if not (0 <= start_iteration <= n_iterations and 0 <= start_subset <= L):
+            raise ValueError("start outside the reconstruction")
+        if start_iteration < n_iterations and start_subset < L:
+            self.reconstruct(events, off[start_subset:], 1, f)
+            start_iteration += 1
+        if start_iteration < n_iterations:
+            self.reconstruct(events, off, n_iterations - start_iteration, f)
+
     def reconstruct_host(self, events, offsets, n_iterations, f):
         """Host events + host f (in/out); H2D streaming overlapped with projection."""
         n = (events.numel() if hasattr(events, "numel") else np.asarray(events).size) // 6

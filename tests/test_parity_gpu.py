@@ -900,3 +900,37 @@ def test_watchdog_aborts_stalled_combine(pkg, monkeypatch):
     rec.close()  # aborts the communicator; the stall exits on the abort flag
     print(f"[watchdog] destroy (ncclCommAbort) took {time.time() - t1:.2f} s")
     assert time.time() - t1 < 3.0
+
+
+def test_checkpoint_and_resume(pkg):
+    """SURVEY.md §5 checkpoint / resume: the state between subsets is f alone (PAPER.md lines
+    466-468). A C1 reconstruction of 2 iterations stopped after subset 0 of iteration 1 (f
+    copied out = the checkpoint) and resumed with Reconstructor.resume in a NEW context
+    equals the uninterrupted reconstruction and the oracle's."""
+    cfg, ev, s = inputs("C1")
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    d_ev = dev(ev)
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f_full = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(d_ev, off, 2, f_full)
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.reconstruct(d_ev, off, 1, f)           # iteration 0
+    rec.reconstruct(d_ev, off[:2], 1, f)       # iteration 1, subset 0 -> checkpoint
+    rec.synchronize()
+    ckpt = f.cpu().numpy().copy()
+    rec.close()
+    rec2 = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+    f2 = dev(ckpt)
+    rec2.resume(d_ev, off, 2, f2, start_iteration=1, start_subset=1)
+    rec2.synchronize()
+    rec2.close()
+    got = f2.cpu().numpy().astype(np.float64)
+    np.testing.assert_allclose(got, f_full.cpu().numpy().astype(np.float64), rtol=1e-5, atol=0)
+    ref = oracle.reconstruct(oracle.geom(cfg.dims, cfg.voxel_mm), ev, off, 2, s, np.ones(cfg.n_voxels))
+    assert rel_l2(got, ref) <= REL_L2_RECON
+    with pytest.raises(ValueError):
+        rec2 = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
+        try:
+            rec2.resume(d_ev, off, 2, f2, start_iteration=3, start_subset=0)
+        finally:
+            rec2.close()
