@@ -524,6 +524,7 @@ def main():
         roof_sec = {"bound": "l2_sectors_two_pass", "achieved": sectors / proj_avg_s, "peak": sectors / t_ceil,
                     "unit": "sectors/s", "frac": t_ceil / proj_avg_s, "sectors_per_launch": sectors,
                     "path_elements_per_sector": 2 * pairs / sectors,
+                    "sector_overfetch": 32.0 * sectors / alg_l2_bytes,
                     "what": "ncu L2 sectors of one subset's z-slab launches (gathers in pass A, REDs in pass B) / live "
                             "projection time, vs the two-pass ceiling gathers / random-gather rate + REDs / random-RED "
                             "rate (live L2 microbenchmarks)"}
@@ -535,9 +536,11 @@ def main():
         roof_sec = {"bound": "l2_sectors", "achieved": sectors / proj_avg_s, "peak": peak_sec, "unit": "sectors/s",
                     "frac": sectors / proj_avg_s / peak_sec, "sectors_per_launch": sectors,
                     "path_elements_per_sector": 2 * pairs / sectors,
+                    "sector_overfetch": 32.0 * sectors / alg_l2_bytes,
                     "what": "ncu L2 sectors of k_project (gathers + REDs, profiles/r02_traffic.json) / live duration, "
                             "vs the max sector rate over the live L2 microbenchmark modes (random RED, random gather, "
-                            "random / 8-lane / 32-lane gather+RED pairs)"}
+                            "random / 8-lane / 32-lane gather+RED pairs); sector_overfetch = 32 B x sectors / "
+                            "algorithmic bytes (4 B gather + 4 B RED per path element, 24 B per event)"}
     # request view (DESIGN.md §7 summary): the SM->L2 request interface takes about one request
     # cycle per SM clock; a gather request (any sectors of one 128-byte line) costs one cycle,
     # a RED one cycle per 32-byte sector (tools/request_probe.cu)
