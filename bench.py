@@ -497,7 +497,9 @@ def main():
             sectors = tr["l2_sectors_read_per_launch"] + tr["l2_sectors_red_per_launch"]
     except (OSError, ValueError, KeyError):
         pass
-    kname = ("k_project<0> (fused Siddon + forward + back-projection)" if n_slabs == 1 else
+    wide = ev_per_launch >= int(os.environ.get("LMOSEM_WIDE_N", "400000"))  # the library's MODE 6 rule
+    kname = ((f"k_project<{6 if wide else 5}> (fused Siddon + forward + back-projection, texture gathers, "
+              f"{'224 x 4' if wide else '256 x 3'} threads x CTAs per SM)") if n_slabs == 1 else
              f"k_project<2>/<3> (z-slab form: {n_slabs} forward-projection + {n_slabs} back-projection launches per "
              f"subset, summed)")
     roof = {"kernel": kname, "bound": "l2",
