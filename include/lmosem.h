@@ -31,10 +31,11 @@
  *  - Distribution (§III.A; §IV.A): with
  *    world > 1, subset_step / reconstruct are collective. Every rank passes the WHOLE
  *    subset; rank r projects the block [floor(r*N/P), floor((r+1)*N/P)) (block
- *    distribution), f is replicated (copy distribution) and c is combined by NCCL
- *    (copy(add)): by default reduce-scatter + block update + all-gather (the paper's
- *    PSD -> ISD switch), or all-reduce + full update (lmosem_set_combine). Either way the
- *    replicas of f are identical on return.
+ *    distribution), f is replicated (copy distribution) and c is combined over NVLink
+ *    (copy(add)) by the paper's PSD -> ISD switch — reduce-scatter, block update,
+ *    all-gather — as one fused multimem kernel when available (else NCCL collectives), or
+ *    by an all-reduce + full update (lmosem_set_combine). Either way the replicas of f are
+ *    identical on return. A loopback group (below) emulates the ranks on one GPU.
  *  - Errors: every call returns a status. EINVAL for bad arguments (nothing enqueued),
  *    including a "device" buffer the GPU cannot dereference (pageable host memory;
  *    device, managed and pinned host memory are accepted — cudaPointerGetAttributes);
@@ -145,7 +146,8 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  * when world > 1; else ALLREDUCE. EINVAL for other values. */
 #define LMOSEM_COMBINE_ALLREDUCE 1
 #define LMOSEM_COMBINE_ISD 2
-/* LMOSEM_COMBINE_FUSED (opt-in): the ISD switch as ONE kernel over
+/* LMOSEM_COMBINE_FUSED (automatic for world > 1 when multimem is
+ * available and the self-test passed, see above): the ISD switch as ONE kernel over
  * NVLink peer memory (NCCL 2.28 symmetric windows + device communicator): rank r reads its
  * block of c summed over ranks (multimem.ld_reduce in the NVSwitch when available, else
  * peer loads), updates it and writes the new f block to every rank (multimem.st or peer
