@@ -99,6 +99,8 @@ typedef struct {
                               kernel (also re-zeroes c); ISD / FUSED the brick -> caller-layout
                               copy of f (written on the last subset of a reconstruct) */
     double h2d_ms;         /* event uploads in lmosem_reconstruct_host (copy stream) */
+    double tune_fused_ms;  /* world > 1: ms per combine of the fused kernel and of ISD, timed on */
+    double tune_isd_ms;    /* this box at init (max over the ranks; 0 = not timed), see below */
 } lmosem_stats;
 
 /* Library version as "lmosem <major>.<minor> sm_100a". */
@@ -141,13 +143,15 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  *     l.15-19): ncclReduceScatter(c) gives rank r the sum over its contiguous block of the
  *     internal image, rank r updates only that block (1/P of step 2), ncclAllGather
  *     rebuilds the full f on every rank. Same NVLink bytes, 1/P of the update work.
- * 0 (default) = FUSED when world > 1 over NCCL, the LSA team has multimem (NVLS) and the
- * fused kernel passed its self-test at init (set LMOSEM_AUTO_FUSED=0 to skip it); else ISD
- * when world > 1; else ALLREDUCE. EINVAL for other values. */
+ * 0 (default) = for world > 1 over NCCL: the fused combine is set up and self-tested at
+ * init, then it and ISD are each timed on this box (lmosem_stats.tune_*_ms, max over the
+ * ranks) and the faster is the automatic combine; ISD when the fused one cannot be set up or
+ * fails its self-test, or with LMOSEM_AUTO_FUSED=0. ALLREDUCE for world == 1. EINVAL for
+ * other values. */
 #define LMOSEM_COMBINE_ALLREDUCE 1
 #define LMOSEM_COMBINE_ISD 2
-/* LMOSEM_COMBINE_FUSED (automatic for world > 1 when multimem is
- * available and the self-test passed, see above): the ISD switch as ONE kernel over
+/* LMOSEM_COMBINE_FUSED (automatic for world > 1 when it passes its
+ * self-test and times faster than ISD, see above): the ISD switch as ONE kernel over
  * NVLink peer memory (NCCL 2.28 symmetric windows + device communicator): rank r reads its
  * block of c summed over ranks (multimem.ld_reduce in the NVSwitch when available, else
  * peer loads), updates it and writes the new f block to every rank (multimem.st or peer

@@ -1035,6 +1035,79 @@ lmosem_status setup_fused(lmosem_ctx* ctx) {
     return LMOSEM_OK;
 }
 
+// Times the two P > 1 combines on this box (collective; run at init after the fused
+// combine's self-test): 2 warm-up and 5 timed runs of the fused kernel and of reduce-scatter
+// + block update + all-gather on the context's own images (zero at init, zero again after),
+// the max over the ranks of each, in ctx->st.tune_fused_ms / tune_isd_ms (ms per combine).
+lmosem_status tune_combine(lmosem_ctx* ctx) {
+    const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
+    int64_t blk_b, blk_e, alloc;
+    isd_block(ctx->bricks.nb, ctx->rank, ctx->world, &blk_b, &blk_e, &alloc);
+    cudaEvent_t ev[2] = {nullptr, nullptr};
+    float* d_t = nullptr;
+    lmosem_status s = LMOSEM_OK;
+    float t[2] = {0.f, 0.f};
+    auto run = [&](int which) -> lmosem_status {
+        if (which == 0) return coll_fused(ctx, chunk);
+        lmosem_status r;
+        if ((r = coll_reduce_scatter(ctx, ctx->c, ctx->c + 8 * b0, (size_t)(8 * chunk)))) return r;
+        if ((r = launch_update(ctx, nullptr, blk_b, blk_e, alloc))) return r;
+        return coll_all_gather(ctx, ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk));
+    };
+    do {
+        if (cudaEventCreate(&ev[0]) != cudaSuccess || cudaEventCreate(&ev[1]) != cudaSuccess ||
+            cudaMalloc(&d_t, 2 * sizeof(float)) != cudaSuccess) {
+            s = fail(ctx, LMOSEM_ECUDA, "tune_combine: events / buffer");
+            break;
+        }
+        for (int which = 0; which < 2 && !s; ++which) {
+            for (int i = 0; i < 2 && !s; ++i) s = run(which);
+            if (s) break;
+            not_kernel(ctx);
+            if (cudaEventRecord(ev[0], ctx->stream) != cudaSuccess) {
+                s = fail(ctx, LMOSEM_ECUDA, "tune_combine: record");
+                break;
+            }
+            for (int i = 0; i < 5 && !s; ++i) s = run(which);
+            if (s) break;
+            not_kernel(ctx);
+            if (cudaEventRecord(ev[1], ctx->stream) != cudaSuccess) {
+                s = fail(ctx, LMOSEM_ECUDA, "tune_combine: record");
+                break;
+            }
+            if ((s = wait_done(ctx, nullptr, ev[1]))) break;
+            float ms = 0.f;
+            cudaEventElapsedTime(&ms, ev[0], ev[1]);
+            t[which] = ms / 5.f;
+        }
+        if (s) break;
+        // agree on the times: max over the ranks
+        not_kernel(ctx);
+        if (cudaMemcpyAsync(d_t, t, sizeof(t), cudaMemcpyHostToDevice, ctx->stream) != cudaSuccess) {
+            s = fail(ctx, LMOSEM_ECUDA, "tune_combine: copy");
+            break;
+        }
+        if (ncclAllReduce(d_t, d_t, 2, ncclFloat32, ncclMax, ctx->comm, ctx->stream) != ncclSuccess) {
+            s = fail(ctx, LMOSEM_ENCCL, "tune_combine: ncclAllReduce");
+            break;
+        }
+        if (cudaMemcpyAsync(t, d_t, sizeof(t), cudaMemcpyDeviceToHost, ctx->stream) != cudaSuccess ||
+            cudaMemsetAsync(ctx->c, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream) != cudaSuccess ||
+            cudaMemsetAsync(ctx->fb, 0, sizeof(float) * 8 * ctx->nb_alloc, ctx->stream) != cudaSuccess) {
+            s = fail(ctx, LMOSEM_ECUDA, "tune_combine: copy back");
+            break;
+        }
+        s = wait_done(ctx, ctx->stream);
+    } while (false);
+    for (auto e : ev)
+        if (e) cudaEventDestroy(e);
+    if (d_t) cudaFree(d_t);
+    if (s) return s;
+    ctx->st.tune_fused_ms = t[0];
+    ctx->st.tune_isd_ms = t[1];
+    return LMOSEM_OK;
+}
+
 }  // namespace
 
 namespace {
@@ -1236,15 +1309,22 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     }
     cuda(cudaStreamSynchronize(ctx->stream), "sync");
     if (s != LMOSEM_OK) return bail(s);
-    // world > 1 over NCCL: set up the fused combine (NEXT-1) and self-test it; it becomes the
-    // automatic combine when the LSA team has multimem (NVLS). Otherwise, or with
-    // LMOSEM_AUTO_FUSED=0, the automatic combine is ISD (reduce-scatter + all-gather).
-    if (ctx->comm && world > 1) {
+    // world > 1 over NCCL: set up the fused combine (NEXT-1) and self-test it (ISD, i.e.
+    // reduce-scatter + all-gather, stays automatic when it fails or with LMOSEM_AUTO_FUSED=0).
+    // If it sets up and passes, both combines are timed on this box (tune_combine) and the
+    // faster one becomes the automatic combine. LMOSEM_AUTO_FUSED=force does the same on a
+    // 1-rank communicator (tests).
+    {
         const char* af = std::getenv("LMOSEM_AUTO_FUSED");
-        if (!(af && af[0] == '0')) {
+        const bool force = af && std::strcmp(af, "force") == 0;
+        if (ctx->comm && (world > 1 || force) && !(af && af[0] == '0')) {
             const lmosem_status fs = setup_fused(ctx);
             if (ctx->failed) return bail(fs);
-            if (fs == LMOSEM_OK && ctx->dev_comm_mm) ctx->auto_combine = LMOSEM_COMBINE_FUSED;
+            if (fs == LMOSEM_OK) {
+                const lmosem_status ts = tune_combine(ctx);
+                if (ts) return bail(ts);
+                ctx->auto_combine = ctx->st.tune_fused_ms <= ctx->st.tune_isd_ms ? LMOSEM_COMBINE_FUSED : LMOSEM_COMBINE_ISD;
+            }
         }
     }
     if (loop) {  // join the group: one context per rank, all on the group's device

@@ -934,3 +934,23 @@ def test_checkpoint_and_resume(pkg):
             rec2.resume(d_ev, off, 2, f2, start_iteration=3, start_subset=0)
         finally:
             rec2.close()
+
+
+def test_combine_autotune_at_init(pkg, monkeypatch):
+    """The automatic P > 1 combine is chosen by timing (include/lmosem.h): after the fused
+    combine's self-test, init times it and ISD on this box and keeps the faster. Forced here
+    on a 1-rank communicator (LMOSEM_AUTO_FUSED=force): both times are reported, the choice
+    is one of the two, and the result matches the oracle."""
+    monkeypatch.setenv("LMOSEM_AUTO_FUSED", "force")
+    cfg, ev, s = inputs("C1")
+    rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), dist=(0, 1, pkg.nccl_unique_id()))
+    st = rec.stats()
+    print(f"[autotune] fused {st['tune_fused_ms']:.4f} ms, isd {st['tune_isd_ms']:.4f} ms -> combine {rec.combine}")
+    assert st["tune_fused_ms"] > 0 and st["tune_isd_ms"] > 0
+    assert rec.combine == (3 if st["tune_fused_ms"] <= st["tune_isd_ms"] else 2)
+    f = dev(np.ones(cfg.n_voxels, np.float32))
+    rec.subset_step(dev(ev[:cfg.n_events]), f)
+    rec.synchronize()
+    rec.close()
+    ref = oracle.subset_step(oracle.geom(cfg.dims, cfg.voxel_mm), ev[:cfg.n_events], s, np.ones(cfg.n_voxels))
+    assert maxrel(f.cpu().numpy().astype(np.float64), ref) <= MAXREL_SUBSET
