@@ -126,9 +126,9 @@ lmosem_status lmosem_nccl_unique_id(void* out, size_t size);
 
 /* Creates a context on the current CUDA device.
  *   dims[3]     = {nx, ny, nz} > 0, V < 2^31 (padded internal image < 2^31 floats), and
- *                 at most one extent > 1210: the per-warp path buffer (3 pieces per
+ *                 at most one extent > 1170: the per-warp path buffer (3 pieces per
  *                 dominant-axis slab) must fit in shared memory, so step 1 cuts a longer
- *                 axis into slabs of <= 1210 voxels (lmosem_set_slabs); EINVAL otherwise
+ *                 axis into slabs of <= 1170 voxels (lmosem_set_slabs); EINVAL otherwise
  *   voxel_mm[3] = voxel size in mm, finite and > 0 (float64: the geometry is float64)
  *   norm        = V float32 sensitivity image s (device or host); copied, caller keeps it
  *   dist        = NULL for one GPU, else the rank/world/NCCL id (collective init;
@@ -193,8 +193,8 @@ int32_t lmosem_get_combine(const lmosem_ctx* ctx);
  * slabs of the volume, pass B back-projects slab by slab with the complete fp — so each
  * launch touches one L2-sized image slab. n_slabs = 0 (default) picks the count from a
  * 72 MB-per-slab L2 budget (1 = single fused pass); n_slabs > 0 forces it (clamped to
- * nz/2). The slabs are cut along z, or along the axis longer than 1210 voxels, whose
- * slabs are then never longer than 1210 (at least that many slabs whatever is asked).
+ * nz/2). The slabs are cut along z, or along the axis longer than 1170 voxels, whose
+ * slabs are then never longer than 1170 (at least that many slabs whatever is asked).
  * The result is the same up to fp32 rounding. EINVAL if n_slabs < 0. */
 lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs);
 

@@ -484,8 +484,9 @@ lmosem_status launch_to_row(lmosem_ctx* ctx, float* br, float* row, int zero) {
 }
 
 // Largest clip-box extent (voxels) whose per-warp path buffer (3 pieces per dominant-axis
-// slab, 8 B each, 8 warps per CTA) fits the 227 KB of opt-in shared memory of sm_100a.
-constexpr int kMaxBox = 1210;
+// slab, 8 B each) and clip area (768 B), 8 warps per CTA, fit the 227 KB of opt-in shared
+// memory of sm_100a.
+constexpr int kMaxBox = 1170;
 
 // Largest slab extent along `axis` when it is cut into K even-aligned slabs (slab_geom).
 int max_slab_extent(int n_axis, int K) {
@@ -591,7 +592,7 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
 lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
     const int cap = launch_cap(mode, g);
     const int threads = lmk::proj_threads_of(mode);
-    const size_t sm = (threads / 32) * sizeof(int2) * (size_t)cap;
+    const size_t sm = (threads / 32) * (sizeof(int2) * (size_t)cap + lmk::kClipBytesPerWarp);
     int per_sm = 1;
     lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm);
     if (s) return s;
@@ -1192,8 +1193,12 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     for (int k = 0; k < 3; ++k)
         if (dims[k] > kMaxBox) ctx->slab_axis = k;
     // path buffer of the largest clip box (the whole volume, or a slab of it; see path_cap)
-    ctx->cap = path_cap(std::min(kMaxBox, std::max(dims[0], std::max(dims[1], dims[2]))));
-    ctx->proj_smem = (lmk::PROJ_THREADS / 32) * sizeof(int2) * (size_t)ctx->cap;
+    {  // the largest clip box: the volume with its long axis clamped to kMaxBox (launch_cap's bounds)
+        lmk::GridGeom box = ctx->geom;
+        box.chi[ctx->slab_axis] = std::min(box.chi[ctx->slab_axis], kMaxBox);
+        ctx->cap = launch_cap(0, box);
+    }
+    ctx->proj_smem = (lmk::PROJ_THREADS / 32) * (sizeof(int2) * (size_t)ctx->cap + lmk::kClipBytesPerWarp);
 
     lmosem_status s = LMOSEM_OK;
     auto cuda = [&](cudaError_t e, const char* what) {

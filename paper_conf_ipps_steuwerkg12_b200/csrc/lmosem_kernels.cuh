@@ -29,6 +29,8 @@
 #include <math_constants.h>
 #include <stdint.h>
 
+#include <type_traits>
+
 namespace lmk {
 
 constexpr int HALO_LO = 2;  // padded coordinate p = i + HALO_LO
@@ -54,17 +56,15 @@ constexpr int FIX_BITS = 40;
 #ifndef LMK_APPEND2
 #define LMK_APPEND2 0  // 1: path-buffer prefix from two ballots on n = v0 + v1 + v2 (A/B)
 #endif
-#ifndef LMK_SCALE_PIECES
-#define LMK_SCALE_PIECES 0  // 1: scale every piece length to mm in the geometry loop (A/B)
-#endif
 
-// Per-LOR traversal state (broadcast lane -> warp by shuffles; 16 registers).
+// Per-LOR traversal state (broadcast lane -> warp by shuffles; 14 registers). The piece
+// lengths of the first and last slab (where the clip meets the plane crossings) come from
+// lor_setup in float64, through the warp's shared-memory clip area (k_project).
 struct Lor {
     long long wb0, wc0;  // minor-axis positions at the plane u_a = i0 (Q24.40 voxels, stored frame)
     long long sb, sc;    // their change per slab (stored frame: <= 0)
     float ab, ac;     // crossing offset in a slab: d = g * a (g: distance to the plane, Q.40)
     float lunit;      // mm of chord per unit of u_a
-    float fin, fout;  // clip inside the first / last slab (local coordinate in [0,1])
     int i0, ns;       // first slab index along a, number of slabs
     int code;         // bits 0-1: dominant axis a; 2-3: step of b (1: +1, 3: -1, 0: none); 4-5: c
 };
@@ -84,8 +84,12 @@ __device__ __forceinline__ T sel3(const T (&v)[3], int i) {
 
 // Sets up the traversal of the segment p1 -> p2. Returns false if it contributes
 // nothing (non-finite, zero length, misses the half-open volume).
-__device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const GridGeom& g, Lor& L) {
-    double p1[3], d[3], u1[3], D[3];
+// clip[0..2] / clip[3..5]: the three piece lengths (slab units) of the first / last slab in
+// float64. There the clip (volume entry and exit, segment ends, slab-pass boundaries) meets
+// the plane crossings, and a piece between a clip and a crossing must not be the difference
+// of two rounded floats (a 3.7e-4-slab piece carried 1.5e-4 relative error that way).
+__device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const GridGeom& g, Lor& L, float clip[6]) {
+    double p1[3], d[3], u1[3], D[3], rD[3];
     bool ok = true;
 #pragma unroll
     for (int k = 0; k < 3; ++k) {
@@ -106,8 +110,10 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
 #pragma unroll
     for (int k = 0; k < 3; ++k) {
         const double lo = (double)g.clo[k], hi = (double)g.chi[k];
+        rD[k] = 0.0;
         if (D[k] != 0.0) {
-            double r = 1.0 / D[k];
+            const double r = 1.0 / D[k];
+            rD[k] = r;
             double t0 = (lo - u1[k]) * r, t1 = (hi - u1[k]) * r;
             amin = fmax(amin, fmin(t0, t1));
             amax = fmin(amax, fmax(t0, t1));
@@ -166,8 +172,27 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     L.ab = sb != 0.0 ? isb : 0.0f;
     L.ac = sc != 0.0 ? isc : 0.0f;
     L.lunit = (float)(Lmm * fabs(rDa));
-    L.fin = fminf(fmaxf((float)(ua_in - (double)i0), 0.0f), 1.0f);
-    L.fout = fminf(fmaxf((float)(ua_out - (double)il), 0.0f), 1.0f);
+    {
+        // crossing offsets of the minor axes inside slab i from the exact plane positions, in
+        // the conventions of the fixed-point walk (a position exactly on a plane belongs to
+        // the voxel above it: an up-moving axis crosses one voxel later, a down-moving one at
+        // 0); 1/|s| = |Da / Db| from the clip's reciprocals (no further division)
+        const double fin = fmin(fmax(ua_in - (double)i0, 0.0), 1.0), fout = fmin(fmax(ua_out - (double)il, 0.0), 1.0);
+        const double rb = fabs(Da * sel3(rD, b)), rc = fabs(Da * sel3(rD, c));
+        auto clip_pieces = [&](int i, double dlo, double dhi, float* out) {
+            const double wb = u1b + ((double)i - u1a) * sb, wc = u1c + ((double)i - u1a) * sc;
+            const double gb = wb - floor(wb), gc = wc - floor(wc);
+            const double db = sb > 0.0 ? (1.0 - gb) * rb : (sb < 0.0 ? gb * rb : CUDART_INF);
+            const double dc = sc > 0.0 ? (1.0 - gc) * rc : (sc < 0.0 ? gc * rc : CUDART_INF);
+            const double q1 = fmin(fmax(fmin(db, dc), dlo), dhi), q2 = fmin(fmax(fmax(db, dc), dlo), dhi);
+            out[0] = (float)(q1 - dlo);
+            out[1] = (float)(q2 - q1);
+            out[2] = (float)(dhi - q2);
+        };
+        const bool one = il == i0;
+        clip_pieces(i0, fin, one ? fout : 1.0, clip);
+        clip_pieces(il, one ? fin : 0.0, fout, clip + 3);
+    }
     L.i0 = i0;
     L.ns = il - i0 + 1;
     L.code = a | (sb > 0.0 ? 4 : (sb < 0.0 ? 12 : 0)) | (sc > 0.0 ? 16 : (sc < 0.0 ? 48 : 0));
@@ -197,8 +222,6 @@ __device__ __forceinline__ Lor shfl_lor(const Lor& s, int src) {
     L.ab = __shfl_sync(0xffffffffu, s.ab, src);
     L.ac = __shfl_sync(0xffffffffu, s.ac, src);
     L.lunit = __shfl_sync(0xffffffffu, s.lunit, src);
-    L.fin = __shfl_sync(0xffffffffu, s.fin, src);
-    L.fout = __shfl_sync(0xffffffffu, s.fout, src);
     L.i0 = __shfl_sync(0xffffffffu, s.i0, src);
     L.ns = __shfl_sync(0xffffffffu, s.ns, src);
     L.code = __shfl_sync(0xffffffffu, s.code, src);
@@ -258,10 +281,9 @@ __device__ __forceinline__ Pieces slab_pieces(const Lor& L, const Walk& W, int k
     const int ib = fb ^ W.mb, ic = fc ^ W.mc;  // voxel indices (un-mirrored)
     const float db = fmaf(gb, L.ab, W.bb);  // crossing offsets along u_a in the slab
     const float dc = fmaf(gc, L.ac, W.bc);
-    const float dlo = (k == 0) ? L.fin : 0.0f;
-    const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;
-    const float q1 = fminf(fmaxf(fminf(db, dc), dlo), dhi);
-    const float q2 = fminf(fmaxf(fmaxf(db, dc), dlo), dhi);
+    // no clip here: the first and last slab's lengths are replaced by their float64 values
+    const float q1 = fminf(fminf(db, dc), 1.0f);  // db, dc >= 0
+    const float q2 = fminf(fmaxf(db, dc), 1.0f);
     int Jb0, Jb1, Jc0, Jc1;
     bidx2(W.Ab, W.Bb, W.Db0, W.Db1, ib, Jb0, Jb1);  // halo offsets of b, c are in Ja
     bidx2(W.Ac, W.Bc, W.Dc0, W.Dc1, ic, Jc0, Jc1);
@@ -270,17 +292,11 @@ __device__ __forceinline__ Pieces slab_pieces(const Lor& L, const Walk& W, int k
     P.j0 = Ja + Jb0 + Jc0;
     P.j1 = Ja + ((db <= dc) ? (Jb1 + Jc0) : (Jb0 + Jc1));
     P.j2 = Ja + Jb1 + Jc1;
-#if LMK_SCALE_PIECES
-    P.l0 = (q1 - dlo) * L.lunit;
-    P.l1 = (q2 - q1) * L.lunit;
-    P.l2 = (dhi - q2) * L.lunit;
-#else
     // lengths in units of the slab (u_a); the LOR's mm per unit, lunit, is applied once per
     // LOR to fp and to the back-projected weight (three multiplies fewer per slab)
-    P.l0 = q1 - dlo;
+    P.l0 = q1;
     P.l1 = q2 - q1;
-    P.l2 = dhi - q2;
-#endif
+    P.l2 = 1.0f - q2;
     return P;
 }
 
@@ -337,6 +353,12 @@ __device__ __forceinline__ int2 lds2(unsigned addr) {
     return v;
 }
 
+__device__ __forceinline__ float lds1(unsigned addr) {
+    float v;
+    asm volatile("ld.shared.f32 %0, [%1];" : "=f"(v) : "r"(addr) : "memory");
+    return v;
+}
+
 // path_s: 32-bit shared-window address of the warp's path buffer (8 B per piece).
 __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, const Pieces& P, bool v0, bool v1,
                                         bool v2) {
@@ -377,6 +399,7 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #define LMK_SLAB_MIN_BLOCKS 7  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
+constexpr size_t kClipBytesPerWarp = 32 * 24;  // k_project's clip area: 6 floats per event of a claim
 #ifndef LMK_GEOM_UNROLL
 #define LMK_GEOM_UNROLL 0  // unroll of the geometry loop (0 = the compiler's choice, 2x)
 #endif
@@ -448,6 +471,10 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
     const unsigned path_s = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)wib * cap);
+    // the warp's clip area after all path buffers: per event of its claim, the 6 float64
+    // piece lengths of its first and last slab (lor_setup)
+    const unsigned clip_w = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)(blockDim.x >> 5) * cap) +
+                            (unsigned)wib * (unsigned)kClipBytesPerWarp;
     const unsigned lt = (1u << lane) - 1u;
     // dynamic work distribution: each warp claims consecutive events from a global counter
     // (work[0]; zero at launch), so unequal LOR lengths and small per-rank subsets do not
@@ -516,7 +543,14 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             } else {
                 load_event(events, idx, ev);
             }
-            ok = lor_setup(ev, g, mine);
+            float clip[6];
+            ok = lor_setup(ev, g, mine, clip);
+            if (ok) {
+                const unsigned a = clip_w + 24u * (unsigned)lane;
+                asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a), "f"(clip[0]), "f"(clip[1]) : "memory");
+                asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a + 8u), "f"(clip[2]), "f"(clip[3]) : "memory");
+                asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a + 16u), "f"(clip[4]), "f"(clip[5]) : "memory");
+            }
             if (MODE == 3) {
                 fp_known = fp[idx];
                 ok = ok && fp_known > 0.0f;  // reading S7
@@ -534,7 +568,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         // float64 setup without the traversal (the result is kept live, never stored)
         if (ok) {
             const unsigned h = (unsigned)mine.wb0 ^ (unsigned)mine.wc0 ^ (unsigned)mine.sb ^ (unsigned)mine.sc ^
-                               __float_as_uint(mine.ab + mine.ac + mine.lunit + mine.fin + mine.fout) ^
+                               __float_as_uint(mine.ab + mine.ac + mine.lunit) ^
                                (unsigned)(mine.i0 ^ mine.ns ^ mine.code);
             if (h == 0x9e3779b9u) cb[0] += 1.0f;
         }
@@ -556,13 +590,24 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             int cnt = 0;
             float acc = 0.0f;
             Step S = make_step(L, W, lane);
-#if LMK_GEOM_UNROLL > 0
-#pragma unroll (kGeomUnroll)
-#endif
-            for (int k0 = 0; k0 < L.ns; k0 += 32, advance(S)) {
+            // one 32-slab round: lane l takes slab k0 + l. The first round's lane 0 (slab 0)
+            // and the last round's lane with slab ns - 1 take their float64 clip lengths; the
+            // rounds are peeled so that the middle ones carry no clip test
+            const unsigned clip_l = clip_w + 24u * (unsigned)src;
+            auto round = [&](int k0, auto first, auto last) {
                 const int k = k0 + lane;
                 const bool in = k < L.ns;  // lanes past the last slab compute garbage, store nothing
-                const Pieces P = slab_pieces(L, W, k, S.wb, S.wc, S.Ja);
+                Pieces P = slab_pieces(L, W, k, S.wb, S.wc, S.Ja);
+                if (decltype(first)::value && k == 0) {
+                    P.l0 = lds1(clip_l);
+                    P.l1 = lds1(clip_l + 4u);
+                    P.l2 = lds1(clip_l + 8u);
+                }
+                if (decltype(last)::value && k == L.ns - 1) {
+                    P.l0 = lds1(clip_l + 12u);
+                    P.l1 = lds1(clip_l + 16u);
+                    P.l2 = lds1(clip_l + 20u);
+                }
                 const bool v0 = in && P.l0 > 0.0f, v1 = in && P.l1 > 0.0f, v2 = in && P.l2 > 0.0f;
                 if (kScatter) append3(path_s, cnt, lt, P, v0, v1, v2);
                 if (kGather) {
@@ -578,10 +623,24 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                         acc = fmaf(v2 ? __ldg(fb + P.j2) : 0.f, P.l2, acc);
                     }
                 }
+            };
+            using T_ = std::true_type;
+            using F_ = std::false_type;
+            if (L.ns <= 32) {
+                round(0, T_(), T_());
+            } else {
+                round(0, T_(), F_());
+                advance(S);
+                int k0 = 32;
+#if LMK_GEOM_UNROLL > 0
+#pragma unroll (kGeomUnroll)
+#endif
+                for (; k0 + 32 < L.ns; k0 += 32, advance(S)) round(k0, F_(), F_());
+                round(k0, F_(), T_());
             }
             float fpv = fp_known;
             if (kGather) {
-                fpv = warp_sum(acc) * (LMK_SCALE_PIECES ? 1.0f : L.lunit);
+                fpv = warp_sum(acc) * L.lunit;
                 if (MODE == 1 && lane == 0) fp[base + src] = fpv;
                 if (MODE == 2 && lane == 0) fp[base + src] += fpv;
             } else {
@@ -591,7 +650,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             if (kScatter && fpv > 0.0f) {  // reading S7: skip events with fp <= 0
                 // pass 2: back-projection, lane m <- piece m (path order: consecutive
                 // lanes share 32-byte brick sectors)
-                const float inv = (LMK_SCALE_PIECES ? 1.0f : L.lunit) / fpv;
+                const float inv = L.lunit / fpv;
 #pragma unroll 8
                 for (int m = lane; m < cnt; m += 32) {
                     const int2 q = lds2(path_s + 8u * (unsigned)m);

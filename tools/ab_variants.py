@@ -14,7 +14,6 @@ VARIANTS = {
     "default": [],
     "setup_only": ["LMK_SETUP_ONLY=1"],
     "append2": ["LMK_APPEND2=1"],  # two-ballot path-buffer prefix
-    "scaled": ["LMK_SCALE_PIECES=1"],  # piece lengths scaled to mm in the geometry loop (before r01 end)
     "unroll1": ["LMK_GEOM_UNROLL=1"],
     "unroll3": ["LMK_GEOM_UNROLL=3"],
     "unroll4": ["LMK_GEOM_UNROLL=4"],  # diagnostic: claims + tiles + float64 setup, no traversal

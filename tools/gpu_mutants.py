@@ -21,13 +21,15 @@ H = "lmosem.cu"
 MUTANTS = [
     ("piece 1 from the later crossing", K, "P.j1 = Ja + ((db <= dc) ? (Jb1 + Jc0) : (Jb0 + Jc1));",
      "P.j1 = Ja + ((db <= dc) ? (Jb0 + Jc1) : (Jb1 + Jc0));", False),
-    ("first-slab clip ignored", K, "const float dlo = (k == 0) ? L.fin : 0.0f;", "const float dlo = 0.0f;", False),
-    ("last-slab clip ignored", K, "const float dhi = (k == L.ns - 1) ? L.fout : 1.0f;", "const float dhi = 1.0f;",
-     False),
-    ("fp without mm per slab unit", K, "fpv = warp_sum(acc) * (LMK_SCALE_PIECES ? 1.0f : L.lunit);",
+    ("first-slab float64 clip lengths not used", K, "if (decltype(first)::value && k == 0) {",
+     "if (false && k == 0) {", False),
+    ("last-slab float64 clip lengths not used", K, "if (decltype(last)::value && k == L.ns - 1) {",
+     "if (false && k == L.ns - 1) {", False),
+    ("last slab takes the first slab's clip lengths", K, "P.l0 = lds1(clip_l + 12u);", "P.l0 = lds1(clip_l);", False),
+    ("fp without mm per slab unit", K, "fpv = warp_sum(acc) * L.lunit;",
      "fpv = warp_sum(acc);", False),
     ("back-projected weight without mm per slab unit", K,
-     "const float inv = (LMK_SCALE_PIECES ? 1.0f : L.lunit) / fpv;", "const float inv = 1.0f / fpv;", False),
+     "const float inv = L.lunit / fpv;", "const float inv = 1.0f / fpv;", False),
     ("texture gather of piece 0 reads piece 1's voxel", K,
      "acc = fmaf(v0 ? tex1Dfetch<float>(g.tex_fb, P.j0) : 0.f, P.l0, acc);",
      "acc = fmaf(v0 ? tex1Dfetch<float>(g.tex_fb, P.j1) : 0.f, P.l0, acc);", False),
