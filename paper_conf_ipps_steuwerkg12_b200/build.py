@@ -52,10 +52,10 @@ def build_l2peak() -> str:
 
 
 def build(force: bool = False, verbose: bool = False, defines=(), out: str | None = None,
-          csrc: str | None = None) -> str:
+          csrc: str | None = None, extra=()) -> str:
     """Builds liblmosem.so (and libl2peak.so). `defines`/`out` build an A/B variant of
     the kernels (e.g. defines=["LMK_TRASH=0"], out=".../liblmosem_v.so"); `csrc` compiles
-    a modified copy of the sources (tools/gpu_mutants.py) into `out`."""
+    a modified copy of the sources (tools/gpu_mutants.py) into `out`; `extra` adds nvcc flags."""
     src_dir = csrc or CSRC
     if out is None and not force and not needs_build():
         return SO
@@ -64,7 +64,7 @@ def build(force: bool = False, verbose: bool = False, defines=(), out: str | Non
         build_l2peak()
     inc, lib = nccl_paths()
     tmp = target + f".tmp{os.getpid()}"
-    cmd = [NVCC, *ARCH, "-O3", "-std=c++17", "-lineinfo", "-Xptxas", "-v", *[f"-D{d}" for d in defines],
+    cmd = [NVCC, *ARCH, "-O3", "-std=c++17", "-lineinfo", "-Xptxas", "-v", *[f"-D{d}" for d in defines], *extra,
            "-Xcompiler", "-fPIC,-fvisibility=hidden", "-shared",
            "-I", os.path.join(ROOT, "include"), "-I", src_dir, "-I", inc,
            os.path.join(src_dir, "lmosem.cu"), "-o", tmp,
