@@ -65,7 +65,7 @@ MUTANTS = [
     # the multi-rank combine (round 2: caught by tests/test_loopback_gpu.py, P ranks on one GPU)
     ("combine: events not block-split (every rank projects the whole subset)", H,
      "if (whole_subset) block_range(n, ctx->rank, ctx->world, &b, &e);", "if (false) block_range(n, ctx->rank, ctx->world, &b, &e);", False),
-    ("combine: ISD block offset ignores the rank", H, "b0 = chunk * ctx->rank;", "b0 = 0;", False),
+    ("combine: ISD block offset ignores the rank", H, "b0 = chunk * ctx->rank;", "b0 = 0;", True),
     ("combine: reduce-scatter count in bricks, not floats", H, "coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(8 * chunk))",
      "coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(chunk))", False),
     ("combine: ISD update leaves the other ranks' partial c (no zero_to)", H,
