@@ -69,7 +69,7 @@ MUTANTS = [
     ("combine: reduce-scatter count in bricks, not floats", H, "coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(8 * chunk))",
      "coll_reduce_scatter(ctx, ctx->c, my_c, (size_t)(chunk))", False),
     ("combine: ISD update leaves the other ranks' partial c (no zero_to)", H,
-     "launch_update(ctx, nullptr, blk_b, blk_e, alloc)", "launch_update(ctx, nullptr, blk_b, blk_e)", False),
+     "launch_update(ctx, nullptr, blk_b, blk_e, alloc)", "launch_update(ctx, nullptr, blk_b, blk_e)", True),
     ("combine: ISD all-gather of f dropped", H,
      "        if ((s = coll_all_gather(ctx, ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk)))) return s;\n", "", False),
     ("combine: all-reduce over a brick count", H, "coll_all_reduce(ctx, ctx->c, (size_t)ctx->nbf)",
@@ -105,6 +105,8 @@ def build(only=None):
     for i, (name, fn, old, new, every) in enumerate(names):
         if not _selected(name, only):
             continue
+        if os.environ.get("MUTANTS_KEEP") and os.path.exists(os.path.join(OUT, f"liblmosem_m{i}.so")):
+            continue  # resume a partial build
         d = os.path.join(OUT, f"src{i}")
         shutil.rmtree(d, ignore_errors=True)
         shutil.copytree(CSRC, d)
