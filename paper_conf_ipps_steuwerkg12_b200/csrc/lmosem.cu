@@ -910,7 +910,7 @@ LMOSEM_API int lmosem_debug_trace_reset(void) {
 }
 #endif
 
-LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.4 sm_100a"; }
+LMOSEM_API const char* lmosem_version(void) { return "lmosem 0.5 sm_100a"; }
 
 LMOSEM_API lmosem_status lmosem_block_range(int64_t n, int32_t rank, int32_t world, int64_t* begin, int64_t* end) {
     if (!begin || !end || n < 0 || world < 1 || rank < 0 || rank >= world) return LMOSEM_EINVAL;
