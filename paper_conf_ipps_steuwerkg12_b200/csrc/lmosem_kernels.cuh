@@ -97,10 +97,12 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
         double p2 = (double)ev[3 + k];
         ok = ok && isfinite(p1[k]) && isfinite(p2);
         d[k] = p2 - p1[k];
-        // voxel coordinate by division: a stationary axis' voxel row (a LOR lying in or
-        // near a voxel face) is then decided exactly as the oracle decides it,
-        // floor((p - lo) / v) in float64 (reading S6)
-        u1[k] = (p1[k] - g.lo[k]) / g.v[k];
+        // voxel coordinate: by division on a stationary axis, whose voxel row (a LOR lying
+        // in or near a voxel face) is then decided exactly as the oracle decides it,
+        // floor((p - lo) / v) in float64 (reading S6); a moving axis only needs
+        // the coordinate to rounding (1 ulp moves a crossing by ~1e-16 voxel)
+        u1[k] = (p1[k] - g.lo[k]) * g.inv_v[k];
+        if (d[k] == 0.0) u1[k] = (p1[k] - g.lo[k]) / g.v[k];
         D[k] = d[k] * g.inv_v[k];
     }
     if (!ok) return false;
@@ -133,7 +135,7 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     int i0 = max((int)floor(ua_in), sel3(g.clo, a));
     int il = min((int)ceil(ua_out) - 1, sel3(g.chi, a) - 1);
     if (il < i0) return false;
-    const double rDa = 1.0 / Da;
+    const double rDa = sel3(rD, a);  // 1 / Da from the clip (Da != 0: the dominant axis)
     const double sb = Db * rDa, sc = Dc * rDa;
     const double fx = (double)(1LL << FIX_BITS);
     // Guard: by the clip, the minor positions over the slab range lie in [0, n] up to
@@ -168,17 +170,16 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     }
     // crossing inside a slab: distance g (Q.40 units) to the next plane in the direction
     // of travel, divided by |slope|: d = g * 2^-40 / |s| (no step: never, d = +inf)
-    const float isb = (float)(1.0 / (fabs(sb) * fx)), isc = (float)(1.0 / (fabs(sc) * fx));
-    L.ab = sb != 0.0 ? isb : 0.0f;
-    L.ac = sc != 0.0 ? isc : 0.0f;
+    // 1/|s| = |Da / Db| from the clip's reciprocals (no further division)
+    const double rb = fabs(Da * sel3(rD, b)), rc = fabs(Da * sel3(rD, c));
+    L.ab = sb != 0.0 ? (float)(rb / fx) : 0.0f;
+    L.ac = sc != 0.0 ? (float)(rc / fx) : 0.0f;
     L.lunit = (float)(Lmm * fabs(rDa));
     {
         // crossing offsets of the minor axes inside slab i from the exact plane positions, in
         // the conventions of the fixed-point walk (a position exactly on a plane belongs to
-        // the voxel above it: an up-moving axis crosses one voxel later, a down-moving one at
-        // 0); 1/|s| = |Da / Db| from the clip's reciprocals (no further division)
+        // the voxel above it: an up-moving axis crosses one voxel later, a down-moving one at 0)
         const double fin = fmin(fmax(ua_in - (double)i0, 0.0), 1.0), fout = fmin(fmax(ua_out - (double)il, 0.0), 1.0);
-        const double rb = fabs(Da * sel3(rD, b)), rc = fabs(Da * sel3(rD, c));
         auto clip_pieces = [&](int i, double dlo, double dhi, float* out) {
             const double wb = u1b + ((double)i - u1a) * sb, wc = u1c + ((double)i - u1a) * sc;
             const double gb = wb - floor(wb), gc = wc - floor(wc);

@@ -54,8 +54,8 @@ MUTANTS = [
      "for (int q = lane; q < (3 * m) / 2 - 1; q += 32)", False),
     ("dominant axis not the largest", K, "const int a = (ax >= ay && ax >= az) ? 0 : ((ay >= az) ? 1 : 2);",
      "const int a = (ax >= ay) ? 0 : ((ay >= az) ? 1 : 2);", False),
-    ("voxel row by multiplication with 1/v", K, "u1[k] = (p1[k] - g.lo[k]) / g.v[k];",
-     "u1[k] = (p1[k] - g.lo[k]) * g.inv_v[k];", False),
+    ("stationary-axis voxel row by multiplication with 1/v", K,
+     "        if (d[k] == 0.0) u1[k] = (p1[k] - g.lo[k]) / g.v[k];\n", "", False),
     ("brick voxel order x/y swapped", K, "2 * bx + (q & 1), 2 * by + ((q >> 1) & 1)",
      "2 * bx + ((q >> 1) & 1), 2 * by + (q & 1)", True),
     ("PDL: no wait before the first image access", K, "            pdl_wait();\n            dep_ready = true;",

@@ -1,0 +1,18 @@
+#!/bin/bash
+# Round 2: trimmed LOR setup (reciprocal multiply on moving axes, 1/Da and 1/(s 2^40) from the clip reciprocals) vs the previous tree.
+# (variants/liblmosem_prev.so)
+O=gpurun_out/setup_ab
+mkdir -p $O
+LMOSEM_FUZZ_CASES=1 LMOSEM_FUZZ_SEED0=21081 python -m pytest tests/test_fuzz_gpu.py -q -p no:cacheprovider -k "matches_oracle" 2>&1 | tail -1
+timeout 900 python -m pytest tests -m gpu -x -q -p no:cacheprovider 2>&1 | tail -1
+for rep in 1 2; do
+ for v in prev new; do
+  if [ $v = new ]; then L=""; else L=variants/liblmosem_$v.so; fi
+  for c in C2 C5; do
+   LMOSEM_LIB=$L python bench.py --config $c --no-cpu-baseline --no-e2e --steps 100 > $O/b_${c}_${v}_r$rep.json 2>/dev/null
+   python -c "import json;d=json.load(open('$O/b_${c}_${v}_r$rep.json'));s=d['per_rank_share'];print('$c $v', round(d['ms_per_step'],4), [round(s[k]['project_ms'],4) for k in ('2','4','8')])" 2>&1 | tail -1
+  done
+  LMOSEM_LIB=$L python bench.py --config C4 --steps 10 --no-cpu-baseline --no-e2e > $O/b_C4_${v}_r$rep.json 2>/dev/null
+  python -c "import json;d=json.load(open('$O/b_C4_${v}_r$rep.json'));print('C4 $v', round(d['ms_per_step'],3))" 2>&1 | tail -1
+ done
+done
