@@ -1,7 +1,7 @@
 #!/bin/bash
-# Round 2: trimmed LOR setup (reciprocal multiply on moving axes, 1/Da and 1/(s 2^40) from the clip reciprocals) vs the previous tree.
+# Round 2 A/B vs the previous tree (variants/liblmosem_prev.so): the current change (see the commit).
 # (variants/liblmosem_prev.so)
-O=gpurun_out/setup_ab
+O=gpurun_out/${AB_OUT:-setup_ab}
 mkdir -p $O
 LMOSEM_FUZZ_CASES=1 LMOSEM_FUZZ_SEED0=21081 python -m pytest tests/test_fuzz_gpu.py -q -p no:cacheprovider -k "matches_oracle" 2>&1 | tail -1
 timeout 900 python -m pytest tests -m gpu -x -q -p no:cacheprovider 2>&1 | tail -1
