@@ -468,6 +468,13 @@ def main():
     # every rank releases its context (NCCL communicator) together; rank 0 then runs the
     # single-GPU microbenchmarks and the oracle baseline and prints the line
     n_slabs, rec_combine = rec.slabs, rec.combine
+    st_final = rec.stats()
+    autotune = None
+    if world > 1:  # the library timed the fused combine and ISD at init and kept the faster
+        autotune = {"fused_ms": st_final["tune_fused_ms"], "isd_ms": st_final["tune_isd_ms"],
+                    "chosen": {1: "allreduce", 2: "isd", 3: "fused"}.get(rec_combine),
+                    "what": "ms per combine of each form, timed by lmosem_init on this box (max over ranks); "
+                            "0 = the fused combine could not be set up or failed its self-test"}
     rec.close()
     if world > 1:
         dist.barrier()
@@ -630,6 +637,7 @@ def main():
                                       "of the same loop right after the timed region"},
         "roofline": roof, "roofline_l2_sectors": roof_sec, "roofline_l2_requests": roof_req,
         "roofline_hbm_events": hbm, "roofline_update": upd, "roofline_step": step_roof,
+        "combine_autotune": autotune,
         "p8_share_model": share_model,
         "gpu_launches": launches, "flushed_subset_step": flushed, "per_rank_share": shares,
         "clocks": clocks, "wall_s_timed_region": t_wall,
