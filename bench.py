@@ -472,6 +472,7 @@ def main():
     autotune = None
     if world > 1:  # the library timed the fused combine and ISD at init and kept the faster
         autotune = {"fused_ms": st_final["tune_fused_ms"], "isd_ms": st_final["tune_isd_ms"],
+                    "allreduce_ms": st_final["tune_allreduce_ms"],
                     "chosen": {1: "allreduce", 2: "isd", 3: "fused"}.get(rec_combine),
                     "what": "ms per combine of each form, timed by lmosem_init on this box (max over ranks); "
                             "0 = the fused combine could not be set up or failed its self-test"}

@@ -99,8 +99,9 @@ typedef struct {
                               kernel (also re-zeroes c); ISD / FUSED the brick -> caller-layout
                               copy of f (written on the last subset of a reconstruct) */
     double h2d_ms;         /* event uploads in lmosem_reconstruct_host (copy stream) */
-    double tune_fused_ms;  /* world > 1: ms per combine of the fused kernel and of ISD, timed on */
-    double tune_isd_ms;    /* this box at init (max over the ranks; 0 = not timed), see below */
+    double tune_fused_ms;     /* world > 1: ms per combine of the fused kernel, of ISD and of */
+    double tune_isd_ms;       /* ALLREDUCE, timed on this box at init (max over the ranks; */
+    double tune_allreduce_ms; /* 0 = not timed), see lmosem_set_combine */
 } lmosem_stats;
 
 /* Library version as "lmosem <major>.<minor> sm_100a". */
@@ -144,10 +145,10 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  *     internal image, rank r updates only that block (1/P of step 2), ncclAllGather
  *     rebuilds the full f on every rank. Same NVLink bytes, 1/P of the update work.
  * 0 (default) = for world > 1 over NCCL: the fused combine is set up and self-tested at
- * init, then it and ISD are each timed on this box (lmosem_stats.tune_*_ms, max over the
- * ranks) and the faster is the automatic combine; ISD when the fused one cannot be set up or
- * fails its self-test, or with LMOSEM_AUTO_FUSED=0. ALLREDUCE for world == 1. EINVAL for
- * other values. */
+ * init, then it, ISD and ALLREDUCE are each timed on this box (lmosem_stats.tune_*_ms, max
+ * over the ranks) and the fastest is the automatic combine; ISD when the fused one cannot be
+ * set up or fails its self-test, or with LMOSEM_AUTO_FUSED=0. ALLREDUCE for world == 1.
+ * EINVAL for other values. */
 #define LMOSEM_COMBINE_ALLREDUCE 1
 #define LMOSEM_COMBINE_ISD 2
 /* LMOSEM_COMBINE_FUSED (automatic for world > 1 when it passes its

@@ -1036,10 +1036,10 @@ lmosem_status setup_fused(lmosem_ctx* ctx) {
     return LMOSEM_OK;
 }
 
-// Times the two P > 1 combines on this box (collective; run at init after the fused
-// combine's self-test): 2 warm-up and 5 timed runs of the fused kernel and of reduce-scatter
-// + block update + all-gather on the context's own images (zero at init, zero again after),
-// the max over the ranks of each, in ctx->st.tune_fused_ms / tune_isd_ms (ms per combine).
+// Times the P > 1 combines on this box (collective; run at init after the fused combine's
+// self-test): 2 warm-up and 5 timed runs each of the fused kernel, of reduce-scatter + block
+// update + all-gather (ISD) and of all-reduce + full update, on the context's own images
+// (zero at init, zero again after); the max over the ranks of each in ctx->st.tune_*_ms.
 lmosem_status tune_combine(lmosem_ctx* ctx) {
     const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
     int64_t blk_b, blk_e, alloc;
@@ -1047,21 +1047,25 @@ lmosem_status tune_combine(lmosem_ctx* ctx) {
     cudaEvent_t ev[2] = {nullptr, nullptr};
     float* d_t = nullptr;
     lmosem_status s = LMOSEM_OK;
-    float t[2] = {0.f, 0.f};
+    float t[3] = {0.f, 0.f, 0.f};
     auto run = [&](int which) -> lmosem_status {
         if (which == 0) return coll_fused(ctx, chunk);
         lmosem_status r;
+        if (which == 2) {  // ALLREDUCE: all-reduce of c, then the full update on every rank
+            if ((r = coll_all_reduce(ctx, ctx->c, (size_t)ctx->nbf))) return r;
+            return launch_update(ctx, nullptr);
+        }
         if ((r = coll_reduce_scatter(ctx, ctx->c, ctx->c + 8 * b0, (size_t)(8 * chunk)))) return r;
         if ((r = launch_update(ctx, nullptr, blk_b, blk_e, alloc))) return r;
         return coll_all_gather(ctx, ctx->fb + 8 * b0, ctx->fb, (size_t)(8 * chunk));
     };
     do {
         if (cudaEventCreate(&ev[0]) != cudaSuccess || cudaEventCreate(&ev[1]) != cudaSuccess ||
-            cudaMalloc(&d_t, 2 * sizeof(float)) != cudaSuccess) {
+            cudaMalloc(&d_t, 3 * sizeof(float)) != cudaSuccess) {
             s = fail(ctx, LMOSEM_ECUDA, "tune_combine: events / buffer");
             break;
         }
-        for (int which = 0; which < 2 && !s; ++which) {
+        for (int which = 0; which < 3 && !s; ++which) {
             for (int i = 0; i < 2 && !s; ++i) s = run(which);
             if (s) break;
             not_kernel(ctx);
@@ -1088,7 +1092,7 @@ lmosem_status tune_combine(lmosem_ctx* ctx) {
             s = fail(ctx, LMOSEM_ECUDA, "tune_combine: copy");
             break;
         }
-        if (ncclAllReduce(d_t, d_t, 2, ncclFloat32, ncclMax, ctx->comm, ctx->stream) != ncclSuccess) {
+        if (ncclAllReduce(d_t, d_t, 3, ncclFloat32, ncclMax, ctx->comm, ctx->stream) != ncclSuccess) {
             s = fail(ctx, LMOSEM_ENCCL, "tune_combine: ncclAllReduce");
             break;
         }
@@ -1106,6 +1110,7 @@ lmosem_status tune_combine(lmosem_ctx* ctx) {
     if (s) return s;
     ctx->st.tune_fused_ms = t[0];
     ctx->st.tune_isd_ms = t[1];
+    ctx->st.tune_allreduce_ms = t[2];
     return LMOSEM_OK;
 }
 
@@ -1316,8 +1321,8 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (s != LMOSEM_OK) return bail(s);
     // world > 1 over NCCL: set up the fused combine (NEXT-1) and self-test it (ISD, i.e.
     // reduce-scatter + all-gather, stays automatic when it fails or with LMOSEM_AUTO_FUSED=0).
-    // If it sets up and passes, both combines are timed on this box (tune_combine) and the
-    // faster one becomes the automatic combine. LMOSEM_AUTO_FUSED=force does the same on a
+    // If it sets up and passes, the three combines are timed on this box (tune_combine) and
+    // the fastest becomes the automatic combine. LMOSEM_AUTO_FUSED=force does the same on a
     // 1-rank communicator (tests).
     {
         const char* af = std::getenv("LMOSEM_AUTO_FUSED");
@@ -1328,7 +1333,9 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
             if (fs == LMOSEM_OK) {
                 const lmosem_status ts = tune_combine(ctx);
                 if (ts) return bail(ts);
-                ctx->auto_combine = ctx->st.tune_fused_ms <= ctx->st.tune_isd_ms ? LMOSEM_COMBINE_FUSED : LMOSEM_COMBINE_ISD;
+                const double tf = ctx->st.tune_fused_ms, ti = ctx->st.tune_isd_ms, ta = ctx->st.tune_allreduce_ms;
+                ctx->auto_combine = (tf <= ti && tf <= ta) ? LMOSEM_COMBINE_FUSED
+                                                           : (ti <= ta ? LMOSEM_COMBINE_ISD : LMOSEM_COMBINE_ALLREDUCE);
             }
         }
     }

@@ -47,7 +47,8 @@ class Stats(ctypes.Structure):
     _fields_ = [("launches", ctypes.c_int64), ("subsets", ctypes.c_int64), ("events", ctypes.c_int64),
                 ("timed_subsets", ctypes.c_int64), ("convert_ms", ctypes.c_double), ("project_ms", ctypes.c_double),
                 ("combine_ms", ctypes.c_double), ("update_ms", ctypes.c_double), ("h2d_ms", ctypes.c_double),
-                ("tune_fused_ms", ctypes.c_double), ("tune_isd_ms", ctypes.c_double)]
+                ("tune_fused_ms", ctypes.c_double), ("tune_isd_ms", ctypes.c_double),
+                ("tune_allreduce_ms", ctypes.c_double)]
 
     def as_dict(self) -> dict:
         return {k: getattr(self, k) for k, _ in self._fields_}

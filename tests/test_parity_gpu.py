@@ -938,16 +938,17 @@ def test_checkpoint_and_resume(pkg):
 
 def test_combine_autotune_at_init(pkg, monkeypatch):
     """The automatic P > 1 combine is chosen by timing (include/lmosem.h): after the fused
-    combine's self-test, init times it and ISD on this box and keeps the faster. Forced here
+    combine's self-test, init times it, ISD and ALLREDUCE on this box and keeps the fastest. Forced here
     on a 1-rank communicator (LMOSEM_AUTO_FUSED=force): both times are reported, the choice
     is one of the two, and the result matches the oracle."""
     monkeypatch.setenv("LMOSEM_AUTO_FUSED", "force")
     cfg, ev, s = inputs("C1")
     rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), dist=(0, 1, pkg.nccl_unique_id()))
     st = rec.stats()
-    print(f"[autotune] fused {st['tune_fused_ms']:.4f} ms, isd {st['tune_isd_ms']:.4f} ms -> combine {rec.combine}")
-    assert st["tune_fused_ms"] > 0 and st["tune_isd_ms"] > 0
-    assert rec.combine == (3 if st["tune_fused_ms"] <= st["tune_isd_ms"] else 2)
+    tf, ti, ta = st["tune_fused_ms"], st["tune_isd_ms"], st["tune_allreduce_ms"]
+    print(f"[autotune] fused {tf:.4f} ms, isd {ti:.4f} ms, allreduce {ta:.4f} ms -> combine {rec.combine}")
+    assert tf > 0 and ti > 0 and ta > 0
+    assert rec.combine == (3 if tf <= ti and tf <= ta else (2 if ti <= ta else 1))
     f = dev(np.ones(cfg.n_voxels, np.float32))
     rec.subset_step(dev(ev[:cfg.n_events]), f)
     rec.synchronize()
