@@ -146,9 +146,9 @@ lmosem_status lmosem_init(lmosem_ctx** out, const int32_t dims[3], const double 
  *     rebuilds the full f on every rank. Same NVLink bytes, 1/P of the update work.
  * 0 (default) = for world > 1 over NCCL: the fused combine is set up and self-tested at
  * init, then it, ISD and ALLREDUCE are each timed on this box (lmosem_stats.tune_*_ms, max
- * over the ranks) and the fastest is the automatic combine; ISD when the fused one cannot be
- * set up or fails its self-test, or with LMOSEM_AUTO_FUSED=0. ALLREDUCE for world == 1.
- * EINVAL for other values. */
+ * over the ranks) and the fastest is the automatic combine (only ISD and ALLREDUCE are timed
+ * when the fused one cannot be set up or fails its self-test); ISD with LMOSEM_AUTO_FUSED=0.
+ * ALLREDUCE for world == 1. EINVAL for other values. */
 #define LMOSEM_COMBINE_ALLREDUCE 1
 #define LMOSEM_COMBINE_ISD 2
 /* LMOSEM_COMBINE_FUSED (automatic for world > 1 when it passes its

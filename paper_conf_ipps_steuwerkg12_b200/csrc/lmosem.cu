@@ -1040,7 +1040,7 @@ lmosem_status setup_fused(lmosem_ctx* ctx) {
 // self-test): 2 warm-up and 5 timed runs each of the fused kernel, of reduce-scatter + block
 // update + all-gather (ISD) and of all-reduce + full update, on the context's own images
 // (zero at init, zero again after); the max over the ranks of each in ctx->st.tune_*_ms.
-lmosem_status tune_combine(lmosem_ctx* ctx) {
+lmosem_status tune_combine(lmosem_ctx* ctx, bool with_fused) {
     const int64_t chunk = ctx->nb_alloc / ctx->world, b0 = chunk * ctx->rank;
     int64_t blk_b, blk_e, alloc;
     isd_block(ctx->bricks.nb, ctx->rank, ctx->world, &blk_b, &blk_e, &alloc);
@@ -1065,7 +1065,7 @@ lmosem_status tune_combine(lmosem_ctx* ctx) {
             s = fail(ctx, LMOSEM_ECUDA, "tune_combine: events / buffer");
             break;
         }
-        for (int which = 0; which < 3 && !s; ++which) {
+        for (int which = with_fused ? 0 : 1; which < 3 && !s; ++which) {
             for (int i = 0; i < 2 && !s; ++i) s = run(which);
             if (s) break;
             not_kernel(ctx);
@@ -1330,13 +1330,16 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
         if (ctx->comm && (world > 1 || force) && !(af && af[0] == '0')) {
             const lmosem_status fs = setup_fused(ctx);
             if (ctx->failed) return bail(fs);
-            if (fs == LMOSEM_OK) {
-                const lmosem_status ts = tune_combine(ctx);
-                if (ts) return bail(ts);
-                const double tf = ctx->st.tune_fused_ms, ti = ctx->st.tune_isd_ms, ta = ctx->st.tune_allreduce_ms;
-                ctx->auto_combine = (tf <= ti && tf <= ta) ? LMOSEM_COMBINE_FUSED
-                                                           : (ti <= ta ? LMOSEM_COMBINE_ISD : LMOSEM_COMBINE_ALLREDUCE);
-            }
+            // without the fused combine (set-up or self-test failed) ISD and ALLREDUCE are timed
+            const bool fused_ok = fs == LMOSEM_OK;
+            const std::string why = ctx->err;
+            const lmosem_status ts = tune_combine(ctx, fused_ok);
+            if (ts) return bail(ts);
+            ctx->err = why;
+            const double tf = fused_ok ? ctx->st.tune_fused_ms : 1e30, ti = ctx->st.tune_isd_ms,
+                         ta = ctx->st.tune_allreduce_ms;
+            ctx->auto_combine = (tf <= ti && tf <= ta) ? LMOSEM_COMBINE_FUSED
+                                                       : (ti <= ta ? LMOSEM_COMBINE_ISD : LMOSEM_COMBINE_ALLREDUCE);
         }
     }
     if (loop) {  // join the group: one context per rank, all on the group's device
