@@ -592,7 +592,7 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
 lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
     const int cap = launch_cap(mode, g);
     const int threads = lmk::proj_threads_of(mode);
-    const size_t sm = (threads / 32) * (sizeof(int2) * (size_t)cap + lmk::kClipBytesPerWarp);
+    const size_t sm = (threads / 32) * (sizeof(int2) * (size_t)cap + lmk::lor_bytes_per_warp(mode));
     int per_sm = 1;
     lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm);
     if (s) return s;
@@ -1203,7 +1203,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
         box.chi[ctx->slab_axis] = std::min(box.chi[ctx->slab_axis], kMaxBox);
         ctx->cap = launch_cap(0, box);
     }
-    ctx->proj_smem = (lmk::PROJ_THREADS / 32) * (sizeof(int2) * (size_t)ctx->cap + lmk::kClipBytesPerWarp);
+    ctx->proj_smem = (lmk::PROJ_THREADS / 32) * (sizeof(int2) * (size_t)ctx->cap + lmk::lor_bytes_per_warp(0));
 
     lmosem_status s = LMOSEM_OK;
     auto cuda = [&](cudaError_t e, const char* what) {

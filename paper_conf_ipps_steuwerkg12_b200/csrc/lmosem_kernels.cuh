@@ -360,6 +360,38 @@ __device__ __forceinline__ float lds1(unsigned addr) {
     return v;
 }
 
+// The record of a set-up LOR in the warp's LOR area in the z-slab passes: written by its
+// setup lane, read by all 32 lanes with broadcast loads when the warp walks it (4 loads
+// instead of the 16 shuffles of shfl_lor: C4 -1.3 %). wb0 wc0 | sb sc | ab ac lunit i0 |
+// ns code clip0 clip1 | clip2..5. Not in the fused pass: its 4 CTAs per SM would need the
+// 228 KB shared-memory carveout and leave the texture gathers 28 KB of L1 (C2 +17 %;
+// DESIGN.md §7).
+__device__ __forceinline__ void lor_store(unsigned a, const Lor& L, const float clip[6]) {
+    asm volatile("st.shared.v2.b64 [%0], {%1, %2};" ::"r"(a), "l"(L.wb0), "l"(L.wc0) : "memory");
+    asm volatile("st.shared.v2.b64 [%0], {%1, %2};" ::"r"(a + 16u), "l"(L.sb), "l"(L.sc) : "memory");
+    asm volatile("st.shared.v4.b32 [%0], {%1, %2, %3, %4};" ::"r"(a + 32u), "f"(L.ab), "f"(L.ac), "f"(L.lunit),
+                 "r"(L.i0)
+                 : "memory");
+    asm volatile("st.shared.v4.b32 [%0], {%1, %2, %3, %4};" ::"r"(a + 48u), "r"(L.ns), "r"(L.code), "f"(clip[0]),
+                 "f"(clip[1])
+                 : "memory");
+    asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(a + 64u), "f"(clip[2]), "f"(clip[3]), "f"(clip[4]),
+                 "f"(clip[5])
+                 : "memory");
+}
+
+__device__ __forceinline__ Lor lor_load(unsigned a) {
+    Lor L;
+    asm volatile("ld.shared.v2.b64 {%0, %1}, [%2];" : "=l"(L.wb0), "=l"(L.wc0) : "r"(a) : "memory");
+    asm volatile("ld.shared.v2.b64 {%0, %1}, [%2];" : "=l"(L.sb), "=l"(L.sc) : "r"(a + 16u) : "memory");
+    asm volatile("ld.shared.v4.b32 {%0, %1, %2, %3}, [%4];"
+                 : "=f"(L.ab), "=f"(L.ac), "=f"(L.lunit), "=r"(L.i0)
+                 : "r"(a + 32u)
+                 : "memory");
+    asm volatile("ld.shared.v2.b32 {%0, %1}, [%2];" : "=r"(L.ns), "=r"(L.code) : "r"(a + 48u) : "memory");
+    return L;
+}
+
 // path_s: 32-bit shared-window address of the warp's path buffer (8 B per piece).
 __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, const Pieces& P, bool v0, bool v1,
                                         bool v2) {
@@ -400,7 +432,12 @@ __device__ __forceinline__ void append3(unsigned path_s, int& cnt, unsigned lt, 
 #define LMK_SLAB_MIN_BLOCKS 7  // CTAs per SM of the z-slab passes (modes 2, 3)
 #endif
 constexpr int PROJ_THREADS = LMK_CTA_THREADS;
-constexpr size_t kClipBytesPerWarp = 32 * 24;  // k_project's clip area: 6 floats per event of a claim
+// k_project's LOR area, per warp after all path buffers: per event of its claim, the 6
+// float64-derived piece lengths of its first and last slab (24 B), and in the z-slab passes
+// (modes 2, 3) also the 56 B of its Lor (lor_store: 80 B per event)
+constexpr unsigned kLorRecBytes = 80;
+__host__ __device__ constexpr bool lor_in_smem(int mode) { return mode == 2 || mode == 3; }
+__host__ __device__ constexpr size_t lor_bytes_per_warp(int mode) { return 32u * (lor_in_smem(mode) ? kLorRecBytes : 24u); }
 #ifndef LMK_GEOM_UNROLL
 #define LMK_GEOM_UNROLL 0  // unroll of the geometry loop (0 = the compiler's choice, 2x)
 #endif
@@ -472,10 +509,12 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
     const unsigned path_s = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)wib * cap);
-    // the warp's clip area after all path buffers: per event of its claim, the 6 float64
-    // piece lengths of its first and last slab (lor_setup)
-    const unsigned clip_w = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)(blockDim.x >> 5) * cap) +
-                            (unsigned)wib * (unsigned)kClipBytesPerWarp;
+    constexpr bool kLorSmem = lor_in_smem(MODE);
+    constexpr unsigned kRec = kLorSmem ? kLorRecBytes : 24u;  // bytes per event in the LOR area
+    constexpr unsigned kClipOff = kLorSmem ? 56u : 0u;      // its clip lengths in the record
+    // the warp's LOR area after all path buffers (lor_bytes_per_warp)
+    const unsigned lor_w = (unsigned)__cvta_generic_to_shared(smem_path + (size_t)(blockDim.x >> 5) * cap) +
+                           (unsigned)wib * (unsigned)lor_bytes_per_warp(MODE);
     const unsigned lt = (1u << lane) - 1u;
     // dynamic work distribution: each warp claims consecutive events from a global counter
     // (work[0]; zero at launch), so unequal LOR lengths and small per-rank subsets do not
@@ -546,8 +585,10 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             }
             float clip[6];
             ok = lor_setup(ev, g, mine, clip);
-            if (ok) {
-                const unsigned a = clip_w + 24u * (unsigned)lane;
+            if (ok && kLorSmem) {
+                lor_store(lor_w + kRec * (unsigned)lane, mine, clip);
+            } else if (ok) {
+                const unsigned a = lor_w + kRec * (unsigned)lane;
                 asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a), "f"(clip[0]), "f"(clip[1]) : "memory");
                 asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a + 8u), "f"(clip[2]), "f"(clip[3]) : "memory");
                 asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a + 16u), "f"(clip[4]), "f"(clip[5]) : "memory");
@@ -583,7 +624,8 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         while (mask) {
             const int src = __ffs(mask) - 1;
             mask &= mask - 1;
-            const Lor L = shfl_lor(mine, src);
+            const unsigned rec = lor_w + kRec * (unsigned)src;
+            const Lor L = kLorSmem ? lor_load(rec) : shfl_lor(mine, src);
             const Walk W = make_walk(L, g);
             // pass 1: geometry (uniform loop; lanes past the last slab drop their pieces)
             // -> path pieces in shared memory (when back-projecting) and f gathered in the
@@ -594,7 +636,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             // one 32-slab round: lane l takes slab k0 + l. The first round's lane 0 (slab 0)
             // and the last round's lane with slab ns - 1 take their float64 clip lengths; the
             // rounds are peeled so that the middle ones carry no clip test
-            const unsigned clip_l = clip_w + 24u * (unsigned)src;
+            const unsigned clip_l = rec + kClipOff;
             auto round = [&](int k0, auto first, auto last) {
                 const int k = k0 + lane;
                 const bool in = k < L.ns;  // lanes past the last slab compute garbage, store nothing

@@ -26,6 +26,10 @@ MUTANTS = [
     ("last-slab float64 clip lengths not used", K, "if (decltype(last)::value && k == L.ns - 1) {",
      "if (false && k == L.ns - 1) {", False),
     ("last slab takes the first slab's clip lengths", K, "P.l0 = lds1(clip_l + 12u);", "P.l0 = lds1(clip_l);", False),
+    ("z-slab LOR record: slopes b and c swapped on load", K,
+     '"=l"(L.sb), "=l"(L.sc) : "r"(a + 16u)', '"=l"(L.sc), "=l"(L.sb) : "r"(a + 16u)', False),
+    ("z-slab LOR record: clip lengths read 4 bytes off", K, "constexpr unsigned kClipOff = kLorSmem ? 56u : 0u;",
+     "constexpr unsigned kClipOff = kLorSmem ? 52u : 0u;", False),
     ("fp without mm per slab unit", K, "fpv = warp_sum(acc) * L.lunit;",
      "fpv = warp_sum(acc);", False),
     ("back-projected weight without mm per slab unit", K,
