@@ -43,6 +43,10 @@ struct PhaseMarks {
 #define LMOSEM_FUSED_CTAS_PER_SM 4  // fused combine: CTAs (and LSA barriers) per SM
 #endif
 
+#ifndef LMOSEM_ZLIST
+#define LMOSEM_ZLIST 2  // listed z-slab form (lmosem_ctx::zlist_mode)
+#endif
+
 #ifndef LMOSEM_WIDE_N
 // fused launches of >= this many events use the 28-warp shape (MODE 6). Measured on one
 // B200 (profiles/r02_shape_ab): C2 whole subset 0.964 -> 0.947 ms, 1/2 share 0.488 -> 0.487;
@@ -99,6 +103,16 @@ struct lmosem_ctx {
     int slab_axis = 2;         // slabs along z, or along the one axis longer than kMaxBox
     int64_t wide_n = LMOSEM_WIDE_N;  // fused launches of at least this many events run MODE 6 (LMOSEM_WIDE_N)
     float* fp_acc = nullptr;   // per-event forward projections of the z-slab passes
+    // listed z-slab form (k_zclass): per-launch event lists of a subset
+    int zlist_mode = LMOSEM_ZLIST;  // 0: every slab launch runs over all events; 1: coarse lists;
+                                    // 2: + fused launches over fine slabs (LMOSEM_ZLIST)
+    int zfine_per = 2;         // fine slabs per coarse slab (LMOSEM_ZFINE)
+    int zfused_mode = 5;       // k_project mode of the fine-window launches (LMOSEM_ZFUSED_MODE: 5 or 6)
+    int zover = 2;             // fine windows overlap: stride = width / zover (LMOSEM_ZOVER)
+    int* zlist = nullptr;      // lists, zlist_cap indices each
+    int* zcount = nullptr;     // their lengths (kZMaxLists)
+    int64_t zlist_cap = 0;
+    int zlist_n = 0;           // lists allocated
     unsigned long long* work = nullptr;  // k_project work counters (one per launch in a step)
     int work_next = 0;
     int64_t fp_cap = 0;
@@ -567,14 +581,22 @@ int launch_cap(int mode, const lmk::GridGeom& g) {
 }
 
 // Resident CTAs per SM of k_project<mode> with `smem` bytes of path buffers (cached).
-lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks) {
+lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks, bool list = false) {
+    const int key = mode + (list ? 16 : 0);
     for (const auto& o : ctx->occ)
-        if (o.mode == mode && o.smem == smem) {
+        if (o.mode == key && o.smem == smem) {
             *blocks = o.blocks;
             return LMOSEM_OK;
         }
     int b = 0;
-    switch (mode) {
+    if (list) {
+        switch (mode) {
+            case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2, true>, lmk::proj_threads_of(2), smem)); break;
+            case 3: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<3, true>, lmk::proj_threads_of(3), smem)); break;
+            case 5: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<5, true>, lmk::proj_threads_of(5), smem)); break;
+            default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<6, true>, lmk::proj_threads_of(6), smem)); break;
+        }
+    } else switch (mode) {
         case 0: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<0>, lmk::proj_threads_of(0), smem)); break;
         case 1: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<1>, lmk::proj_threads_of(1), smem)); break;
         case 2: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<2>, lmk::proj_threads_of(2), smem)); break;
@@ -584,17 +606,20 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
         default: CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, lmk::k_project<6>, lmk::proj_threads_of(6), smem)); break;
     }
     b = std::max(1, b);
-    ctx->occ.push_back({mode, smem, b});
+    ctx->occ.push_back({key, smem, b});
     *blocks = b;
     return LMOSEM_OK;
 }
 
-lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g) {
+// list != nullptr (MODEs 2, 3, 5, 6): the launch runs over the events list[0 .. *list_n),
+// list_n <= n (on the device; n sizes the grid and the claims)
+lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g,
+                          const int* list = nullptr, const int* list_n = nullptr) {
     const int cap = launch_cap(mode, g);
     const int threads = lmk::proj_threads_of(mode);
     const size_t sm = (threads / 32) * (sizeof(int2) * (size_t)cap + lmk::lor_bytes_per_warp(mode));
     int per_sm = 1;
-    lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm);
+    lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm, list != nullptr);
     if (s) return s;
     const int64_t wpb = threads / 32;
     const int64_t resident = (int64_t)ctx->num_sms * per_sm * wpb;
@@ -611,8 +636,14 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     // guided claims: a full C2/C5 subset (~9 rounds of 32-event claims per warp)
     // gains from the smaller final claims of divisor 3; a rank's share at P >= 2 from 2
     const int gdiv = n >= (int64_t)LMOSEM_GUIDED_ROUNDS * 32 * resident ? LMOSEM_GUIDED_LARGE : LMOSEM_GUIDED_SMALL;
-    void (*k)(const float*, int64_t, const float*, float*, float*, lmk::GridGeom, int, unsigned long long*, int, int);
-    switch (mode) {
+    void (*k)(const float*, int64_t, const float*, float*, float*, lmk::GridGeom, int, unsigned long long*, int, int,
+              const int*, const int*);
+    if (list) switch (mode) {
+        case 2: k = lmk::k_project<2, true>; break;
+        case 3: k = lmk::k_project<3, true>; break;
+        case 5: k = lmk::k_project<5, true>; break;
+        default: k = lmk::k_project<6, true>; break;
+    } else switch (mode) {
         case 0: k = lmk::k_project<0>; break;
         case 1: k = lmk::k_project<1>; break;
         case 2: k = lmk::k_project<2>; break;
@@ -621,7 +652,8 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
         case 5: k = lmk::k_project<5>; break;
         default: k = lmk::k_project<6>; break;
     }
-    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch, gdiv));
+    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch, gdiv, list,
+                list_n));
     return LMOSEM_OK;
 }
 
@@ -632,6 +664,78 @@ lmk::GridGeom slab_geom(const lmosem_ctx* ctx, int k, int K) {
     g.clo[a] = 2 * (int)((int64_t)half * k / K);
     g.chi[a] = (k == K - 1) ? ctx->dims[a] : 2 * (int)((int64_t)half * (k + 1) / K);
     return g;
+}
+
+// The listed z-slab form of step 1: k_zclass sorts the n events into the
+// coarse lists X_k (LORs that leave a fine slab: passes A and B over coarse slab k only for
+// the LORs that meet it) and the fine lists F_j (LORs inside fine slab j: one fused launch
+// over the fine slab box, whose f and c slabs fit L2 together). Order: pass A over every
+// coarse slab (fp of the X LORs complete), then per coarse slab k the fused launches of its
+// fine slabs and pass B of X_k, so c's slab k stays L2-resident across them.
+lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n, int K,
+                                   const std::vector<std::pair<int, int>>& wins) {
+    const int Kf = (int)wins.size();
+    const int nl = K + Kf;
+    if (n > ctx->zlist_cap || nl > ctx->zlist_n) {
+        if (ctx->zlist) CK(cudaFree(ctx->zlist));
+        ctx->zlist = nullptr;
+        ctx->zlist_cap = 0;
+        ctx->zlist_n = 0;
+        CKA(cudaMalloc(&ctx->zlist, sizeof(int) * (size_t)n * nl));
+        ctx->zlist_cap = n;
+        ctx->zlist_n = nl;
+    }
+    if (!ctx->zcount) CKA(cudaMalloc(&ctx->zcount, sizeof(int) * lmk::kZMaxLists));
+    lmk::ZClass zc{};
+    zc.K = K;
+    zc.Kf = Kf;
+    zc.axis = ctx->slab_axis;
+    for (int k = 0; k < K; ++k) {
+        const lmk::GridGeom gk = slab_geom(ctx, k, K);
+        zc.cb[k] = gk.clo[zc.axis];
+        zc.cb[k + 1] = gk.chi[zc.axis];
+    }
+    for (int j = 0; j < Kf; ++j) {
+        zc.wlo[j] = wins[j].first;
+        zc.whi[j] = wins[j].second;
+    }
+    if (Kf > 0) {  // windows j * stride (the last one clamped to end at the axis' end), equal widths
+        zc.ws = Kf > 1 ? (float)wins[1].first : 1.0f;
+        zc.ww = (float)(wins[0].second - wins[0].first);
+        zc.wlast = (float)wins[Kf - 1].first;
+    }
+    not_kernel(ctx);
+    CK(cudaMemsetAsync(ctx->zcount, 0, sizeof(int) * lmk::kZMaxLists, ctx->stream));
+    CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
+    const int zgrid = (int)std::max<int64_t>(1, std::min<int64_t>((n + lmk::kZChunk - 1) / lmk::kZChunk,
+                                                                   (int64_t)ctx->num_sms * 8));
+    CK(launch_k(ctx, lmk::k_zclass, zgrid, lmk::kZThreads, 0, evf, n, ctx->geom, zc, ctx->zlist, ctx->zlist_cap,
+                ctx->zcount));
+    // the first listed launch reads the lists before griddepcontrol.wait: a plain launch
+    ctx->after_kernel = false;
+    const int* X = ctx->zlist;
+    lmosem_status s;
+    for (int k = 0; k < K; ++k)
+        if ((s = launch_mode(ctx, 2, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), X + (size_t)k * ctx->zlist_cap,
+                             ctx->zcount + k)))
+            return s;
+    const int fused = ctx->zfused_mode;
+    for (int k = 0; k < K; ++k) {
+        for (int j = 0; j < Kf; ++j) {
+            const int mid = (zc.wlo[j] + zc.whi[j]) / 2;
+            if (mid < zc.cb[k] || mid >= zc.cb[k + 1]) continue;  // window j runs before pass B of its centre's slab
+            lmk::GridGeom gj = ctx->geom;
+            gj.clo[zc.axis] = zc.wlo[j];
+            gj.chi[zc.axis] = zc.whi[j];
+            if ((s = launch_mode(ctx, fused, evf, n, nullptr, gj, X + (size_t)(K + j) * ctx->zlist_cap,
+                                 ctx->zcount + K + j)))
+                return s;
+        }
+        if ((s = launch_mode(ctx, 3, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), X + (size_t)k * ctx->zlist_cap,
+                             ctx->zcount + k)))
+            return s;
+    }
+    return LMOSEM_OK;
 }
 
 // Step 1 over n device events against ctx->fb (mode 0: accumulate into ctx->c; mode 1:
@@ -658,6 +762,22 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         ctx->fp_cap = 0;
         CKA(cudaMalloc(&ctx->fp_acc, sizeof(float) * n));
         ctx->fp_cap = n;
+    }
+    if (ctx->zlist_mode > 0 && n <= INT32_MAX) {
+        // fine windows along the slab axis (the fused launches gather through the texture
+        // pipe, MODE 5/6): width ~ 1/zfine_per of a coarse slab, stride width/zover, even planes
+        std::vector<std::pair<int, int>> wins;
+        const int na = ctx->dims[ctx->slab_axis];
+        const int W = 2 * std::max(1, na / (2 * K * ctx->zfine_per));
+        const int S = 2 * std::max(1, W / (2 * ctx->zover));
+        if (ctx->zlist_mode == 2 && ctx->geom.tex_fb && W < na) {
+            for (int lo = 0;; lo += S) {
+                const int l = std::min(lo, na - W);
+                wins.push_back({l, l + W});
+                if (l + W >= na) break;
+            }
+        }
+        if (K + (int)wins.size() <= lmk::kZMaxLists) return launch_project_listed(ctx, evf, n, K, wins);
     }
     not_kernel(ctx);
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
@@ -1218,6 +1338,10 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (!cuda(cudaGetDeviceProperties(&prop, ctx->device), "cudaGetDeviceProperties")) return bail(s);
     ctx->num_sms = prop.multiProcessorCount;
     if (const char* e = std::getenv("LMOSEM_PDL")) ctx->pdl = e[0] != '0';  // A/B switch (default on)
+    if (const char* e = std::getenv("LMOSEM_ZLIST")) ctx->zlist_mode = std::max(0, std::min(2, std::atoi(e)));
+    if (const char* e = std::getenv("LMOSEM_ZFINE")) ctx->zfine_per = std::max(1, std::min(8, std::atoi(e)));
+    if (const char* e = std::getenv("LMOSEM_ZFUSED_MODE")) ctx->zfused_mode = std::atoi(e) == 5 ? 5 : 6;
+    if (const char* e = std::getenv("LMOSEM_ZOVER")) ctx->zover = std::max(1, std::min(4, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {
@@ -1243,6 +1367,10 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
         cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
         cuda(cudaFuncSetAttribute(lmk::k_project<5>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
         cuda(cudaFuncSetAttribute(lmk::k_project<6>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<2, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<3, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<5, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        cuda(cudaFuncSetAttribute(lmk::k_project<6, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
     }
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");
@@ -1821,6 +1949,8 @@ LMOSEM_API lmosem_status lmosem_destroy(lmosem_ctx* ctx) {
     if (ctx->norm) cudaFree(ctx->norm);
     if (ctx->scratch) cudaFree(ctx->scratch);
     if (ctx->fp_acc) cudaFree(ctx->fp_acc);
+    if (ctx->zlist) cudaFree(ctx->zlist);
+    if (ctx->zcount) cudaFree(ctx->zcount);
     if (ctx->work) cudaFree(ctx->work);
     if (ctx->own_stream) cudaStreamDestroy(ctx->own_stream);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);

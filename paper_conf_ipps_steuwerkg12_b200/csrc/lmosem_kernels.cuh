@@ -496,12 +496,15 @@ __host__ __device__ constexpr int proj_threads_of(int mode) {
 //         claims per warp).
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
-template <int MODE>
+// LIST (MODEs 2, 3, 5, 6; the listed z-slab form): the launch runs over the events
+// list[0 .. *list_n) (indices into `events` and `fp`, written by k_zclass) instead of [0, n).
+template <int MODE, bool LIST = false>
 __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>()) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap,
                                                              unsigned long long* __restrict__ work, int batch,
-                                                             int gdiv) {
+                                                             int gdiv, const int* __restrict__ list,
+                                                             const int* __restrict__ list_n) {
     constexpr bool kGather = MODE <= 2 || MODE >= 5;  // forward projection in this launch
     constexpr bool kScatter = MODE == 0 || MODE >= 3;  // back-projection
     constexpr bool kTex = MODE >= 5;  // gathers of f through the texture path
@@ -524,6 +527,18 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     // left a tail of that length at the end of every launch
     const int64_t warps_in_grid = (int64_t)gridDim.x * (blockDim.x >> 5);
     int take = batch;
+    // the list and its length were written before the previous launch started (k_zclass
+    // precedes a plain launch), so they are read before griddepcontrol.wait. The host sized
+    // the grid for all events; the claim sizes follow the list's length (lmosem.cu
+    // launch_mode's rule with its defaults: first claims 32 halved while a warp would get
+    // fewer than 4, >= 4; guided divisor 3 from 6 rounds of 32-event claims, else 2)
+    if (LIST) {
+        n = (int64_t)*list_n;
+        take = 32;
+        while (take > 4 && n < (int64_t)take * warps_in_grid * 4) take >>= 1;
+        batch = take;
+        gdiv = n >= 6 * 32 * warps_in_grid ? 3 : 2;
+    }
     pdl_trigger();
     // claims, event tiles and the float64 setup of the first LORs overlap the previous
     // kernel's tail; pass B reads fp during setup, so it waits at once
@@ -554,6 +569,8 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         }
         const int64_t idx = base + lane;
         const bool mine_ev = lane < take && idx < n;
+        // the event (and fp slot) of this lane: idx, or the idx-th listed event
+        const int64_t eidx = LIST ? (mine_ev ? (int64_t)__ldg(list + idx) : 0) : idx;
         // event tile staging: the claimed events (24 B each, contiguous) are loaded with
         // coalesced 16-byte vector loads into the head of the warp's path buffer (idle at
         // this point), then each lane reads its record from shared memory
@@ -564,7 +581,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             take = batch <= 2 ? batch : (int)max((int64_t)2, min((int64_t)batch, g)) & ~1;
         }
         const float* tile_g = events + 6 * base;
-        const bool vec = ((((uintptr_t)tile_g) & 15) == 0) && ((m & 1) == 0);
+        const bool vec = !LIST && ((((uintptr_t)tile_g) & 15) == 0) && ((m & 1) == 0);
         float4* tile_s = reinterpret_cast<float4*>(smem_path + (size_t)wib * cap);
         if (vec) {
             const float4* src = reinterpret_cast<const float4*>(tile_g);
@@ -581,7 +598,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 const float2 a = r[0], b = r[1], c = r[2];
                 ev[0] = a.x; ev[1] = a.y; ev[2] = b.x; ev[3] = b.y; ev[4] = c.x; ev[5] = c.y;
             } else {
-                load_event(events, idx, ev);
+                load_event(events, eidx, ev);
             }
             float clip[6];
             ok = lor_setup(ev, g, mine, clip);
@@ -594,7 +611,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 asm volatile("st.shared.v2.f32 [%0], {%1, %2};" ::"r"(a + 16u), "f"(clip[4]), "f"(clip[5]) : "memory");
             }
             if (MODE == 3) {
-                fp_known = fp[idx];
+                fp_known = fp[eidx];
                 ok = ok && fp_known > 0.0f;  // reading S7
             }
         }
@@ -602,7 +619,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             pdl_wait();
             dep_ready = true;
         }
-        if (MODE == 1 && mine_ev && !ok) fp[idx] = 0.0f;
+        if (MODE == 1 && mine_ev && !ok) fp[eidx] = 0.0f;
         __syncwarp();  // the tile is dead: the path buffer may be overwritten
         unsigned mask = __ballot_sync(0xffffffffu, ok);
 #if LMK_SETUP_ONLY
@@ -684,8 +701,9 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             float fpv = fp_known;
             if (kGather) {
                 fpv = warp_sum(acc) * L.lunit;
-                if (MODE == 1 && lane == 0) fp[base + src] = fpv;
-                if (MODE == 2 && lane == 0) fp[base + src] += fpv;
+                const int64_t esrc = LIST ? (int64_t)__shfl_sync(0xffffffffu, (int)eidx, src) : base + src;
+                if (MODE == 1 && lane == 0) fp[esrc] = fpv;
+                if (MODE == 2 && lane == 0) fp[esrc] += fpv;
             } else {
                 fpv = __shfl_sync(0xffffffffu, fp_known, src);
             }
@@ -702,6 +720,149 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             }
             __syncwarp();
         }
+    }
+}
+
+// ------------------------------------------------------------ listed z-slab form (C4)
+// When the image exceeds L2 the projection runs slab by slab (MODEs 2, 3). k_zclass sorts
+// each event of the subset, once, into the launches that need it ("Listed
+// z-slab form"). The slab-axis range [zl, zh] of its chord clipped to the volume (float32
+// against a grown box, zclass_bits) decides:
+//   - inside fine window j (the first one), kZMarginF voxels clear of its planes: fine list
+//     F_j. Such a LOR's pieces are those of the whole-volume clip, so one fused launch
+//     (MODE 5/6) over the window's box projects it completely; a window's f and c fit L2
+//     together. Windows may overlap (stride < width: more LORs fit one);
+//   - else: coarse list X_k of every coarse slab k that [zl - m, zh + m] meets (passes A
+//     and B over slab k; a listed LOR that misses the slab is dropped by its clip).
+// An event that cannot contribute (non-finite, zero length, missing the volume) is in no
+// list. Lists: lists + l * cap, lengths counts[l]; l < K coarse, K <= l < K + Kf fine.
+constexpr int kZMaxLists = 32;
+struct ZClass {
+    int K, Kf, axis;
+    int cb[kZMaxLists + 1];  // coarse slab planes (voxels along axis): cb[0] = 0 .. cb[K] = n
+    int wlo[kZMaxLists], whi[kZMaxLists];  // fine windows [wlo, whi): wlo = j * ws (the last
+    float ws, ww, wlast;                   // one: wlast), whi = wlo + ww
+};
+
+// Membership bits of one event (bit l set: the event goes to list l), in float32 against a
+// box grown by kZMarginF voxels, so the clipped range contains the float64 one (lor_setup)
+// up to float32 rounding (< 1e-2 voxel while both ends lie within 2 volume extents of the
+// centre; farther or non-finite LORs go to every coarse list, where lor_setup decides):
+//   - a LOR is fine-local only kZMarginF clear of its window's planes;
+//   - a coarse list gets every LOR whose grown range meets the slab (a superset);
+//   - no list: clearly zero length or missing the grown box.
+constexpr float kZMarginF = 0.02f;
+__device__ __forceinline__ unsigned zclass_bits(const float ev[6], const GridGeom& g, const ZClass& zc) {
+    constexpr float m = kZMarginF;
+    const unsigned all = (1u << zc.K) - 1u;
+    const float nmax = (float)max(g.n[0], max(g.n[1], g.n[2]));
+    float u1[3], D[3];
+    bool far = false, zero = true;
+#pragma unroll
+    for (int k = 0; k < 3; ++k) {
+        const float lo = (float)g.lo[k], iv = (float)g.inv_v[k], c = 0.5f * (float)g.n[k];
+        const float a = (ev[k] - lo) * iv, b = (ev[3 + k] - lo) * iv;
+        far = far || !(fabsf(a - c) <= 2.0f * nmax && fabsf(b - c) <= 2.0f * nmax);  // also NaN / inf
+        zero = zero && ev[k] == ev[3 + k];
+        u1[k] = a;
+        D[k] = b - a;
+    }
+    if (far) return all;
+    if (zero) return 0u;  // p1 == p2: zero length (exactly as lor_setup decides)
+    float amin = 0.0f, amax = 1.0f;
+#pragma unroll
+    for (int k = 0; k < 3; ++k) {
+        const float hi = (float)g.n[k] + m;
+        if (ev[k] != ev[3 + k]) {
+            // approximate reciprocal: its error (~1 ulp; 1/0 = inf drops the axis' bound)
+            // only lengthens or shortens the grown clip far inside the margin
+            float r;
+            asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(D[k]));
+            const float t0 = (-m - u1[k]) * r, t1 = (hi - u1[k]) * r;
+            amin = fmaxf(amin, fminf(t0, t1));
+            amax = fminf(amax, fmaxf(t0, t1));
+        } else if (u1[k] < -m || u1[k] > hi) {
+            return 0u;  // parallel to axis k, clearly outside
+        }
+    }
+    if (!(amax >= amin)) return 0u;
+    const float us = sel3(u1, zc.axis), Ds = sel3(D, zc.axis);
+    const float za = fmaf(amin, Ds, us), zb = fmaf(amax, Ds, us);
+    const float zl = fminf(za, zb), zh = fmaxf(za, zb);
+    if (!isfinite(zl) || !isfinite(zh)) return all;
+    if (zc.Kf > 0) {
+        // the window starting last at or below zl - m is the only candidate (earlier ones
+        // end earlier), and the clamped last window
+        const int j = min((int)floorf(fmaxf(zl - m, 0.0f) / zc.ws), zc.Kf - 1);
+        const float lo = j == zc.Kf - 1 ? zc.wlast : (float)j * zc.ws;
+        if (zl >= lo + m && zh <= lo + zc.ww - m) return 1u << (zc.K + j);
+        if (j > 0 && j == zc.Kf - 1) {  // the last window may start below the stride grid
+            const float lo2 = (float)(j - 1) * zc.ws;
+            if (zl >= lo2 + m && zh <= lo2 + zc.ww - m) return 1u << (zc.K + j - 1);
+        }
+    }
+    unsigned bits = 0u;
+    for (int k = 0; k < zc.K; ++k)
+        if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) bits |= 1u << k;
+    return bits;
+}
+
+// One CTA per chunk of kZChunk consecutive events (grid-stride): the appends are counted per
+// warp in shared memory, then one global atomic per list and chunk reserves the chunk's
+// range (a global atomic per warp and list serialised on the K + Kf counters: 0.6-1.5 ms
+// per C4 subset). Within a list the events keep chunk order, within a chunk warp order.
+constexpr int kZThreads = 256, kZPer = 8, kZChunk = kZThreads * kZPer;
+__global__ void __launch_bounds__(kZThreads) k_zclass(const float* __restrict__ events, int64_t n, GridGeom g,
+                                                      ZClass zc, int* __restrict__ lists, int64_t cap,
+                                                      int* __restrict__ counts) {
+    pdl_wait();
+    pdl_trigger();
+    __shared__ int s_cnt[kZMaxLists], s_base[kZMaxLists];
+    __shared__ int s_woff[kZThreads / 32][kZPer][kZMaxLists];
+    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+    const unsigned lt = (1u << lane) - 1u;
+    const int nl = zc.K + zc.Kf;
+    for (int64_t c0 = (int64_t)blockIdx.x * kZChunk; c0 < n; c0 += (int64_t)gridDim.x * kZChunk) {
+        if ((int)threadIdx.x < nl) s_cnt[threadIdx.x] = 0;
+        __syncthreads();
+        unsigned bits[kZPer];
+        // all kZPer events' loads in flight before the float64 clips
+        float ev[kZPer][6];
+#pragma unroll
+        for (int p = 0; p < kZPer; ++p) {
+            const int64_t i = c0 + p * kZThreads + threadIdx.x;
+            load_event(events, i < n ? i : n - 1, ev[p]);
+        }
+#pragma unroll
+        for (int p = 0; p < kZPer; ++p)
+            bits[p] = c0 + p * kZThreads + threadIdx.x < n ? zclass_bits(ev[p], g, zc) : 0u;
+#pragma unroll
+        for (int p = 0; p < kZPer; ++p) {
+            unsigned any = __reduce_or_sync(0xffffffffu, bits[p]);
+            while (any) {
+                const int l = __ffs(any) - 1;
+                any &= any - 1;
+                const unsigned mask = __ballot_sync(0xffffffffu, (bits[p] >> l) & 1u);
+                if (lane == 0) s_woff[w][p][l] = atomicAdd(&s_cnt[l], __popc(mask));
+            }
+        }
+        __syncthreads();
+        if ((int)threadIdx.x < nl) s_base[threadIdx.x] = s_cnt[threadIdx.x] ? atomicAdd(counts + threadIdx.x, s_cnt[threadIdx.x]) : 0;
+        __syncthreads();
+#pragma unroll
+        for (int p = 0; p < kZPer; ++p) {
+            unsigned any = __reduce_or_sync(0xffffffffu, bits[p]);
+            while (any) {
+                const int l = __ffs(any) - 1;
+                any &= any - 1;
+                const bool in = (bits[p] >> l) & 1u;
+                const unsigned mask = __ballot_sync(0xffffffffu, in);
+                if (in)
+                    lists[(int64_t)l * cap + s_base[l] + s_woff[w][p][l] + __popc(mask & lt)] =
+                        (int)(c0 + p * kZThreads + threadIdx.x);
+            }
+        }
+        __syncthreads();  // s_cnt / s_woff are rewritten by the next chunk
     }
 }
 
