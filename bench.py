@@ -493,14 +493,19 @@ def main():
     # image (V floats), or in the z-slab form one slab of the brick image (L2-resident)
     l2_floats = cfg.n_voxels if n_slabs == 1 else nbf // n_slabs
     l2 = l2_peak_gbs(l2_floats, nbf)
-    # 4 B gather + 4 B RED per path element, 24 B per event and read (the z-slab form reads
-    # the events in each of its 2 x n_slabs launches)
-    alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)
-    traffic, sectors = None, None
+    # the listed z-slab form (library default for images beyond L2: k_zclass lists, passes A/B
+    # over the coarse slabs for the LORs that cross them, fused launches over fine windows)
+    listed = n_slabs > 1 and os.environ.get("LMOSEM_ZLIST", "2") != "0"
+    ev_reads = 1 if (n_slabs == 1 or listed) else 2 * n_slabs
+    # 4 B gather + 4 B RED per path element, 24 B per event and read (the unlisted z-slab form
+    # reads the events in each of its 2 x n_slabs launches; the listed form counts them once)
+    alg_l2_bytes = pairs * 8.0 + ev_per_launch * 24.0 * ev_reads
+    traffic, sectors, tr = None, None, None
     try:
         with open(os.path.join(ROOT, "profiles", "r02_traffic.json")) as fh:
             tr = json.load(fh).get(name)
-        if tr and tr.get("launches_per_step", 1) == (2 * n_slabs if n_slabs > 1 else 1):
+        form_ok = tr and (tr.get("form") == "listed") == listed
+        if form_ok and (listed or tr.get("launches_per_step", 1) == (2 * n_slabs if n_slabs > 1 else 1)):
             traffic = tr["dram_bytes_read_per_launch"] + tr["dram_bytes_write_per_launch"]
             sectors = tr["l2_sectors_read_per_launch"] + tr["l2_sectors_red_per_launch"]
     except (OSError, ValueError, KeyError):
@@ -508,6 +513,9 @@ def main():
     wide = ev_per_launch >= int(os.environ.get("LMOSEM_WIDE_N", "400000"))  # the library's MODE 6 rule
     kname = ((f"k_project<{6 if wide else 5}> (fused Siddon + forward + back-projection, texture gathers, "
               f"{'224 x 4' if wide else '256 x 3'} threads x CTAs per SM)") if n_slabs == 1 else
+             (f"k_project<2,list>/<5,list>/<3,list> (listed z-slab form: k_zclass, then {n_slabs} forward-projection "
+              f"launches over the LORs crossing each coarse slab, fused launches over overlapping fine windows for the "
+              f"LORs inside one, {n_slabs} back-projection launches; summed per subset)") if listed else
              f"k_project<2>/<3> (z-slab form: {n_slabs} forward-projection + {n_slabs} back-projection launches per "
              f"subset, summed)")
     roof = {"kernel": kname, "bound": "l2",
@@ -526,7 +534,7 @@ def main():
         roof["frac_vs_random_pairs"] = roof["achieved"] / (l2["pair"] * 8.0 / 1e9)
         roof["l2_micro_ops_per_s"] = l2
     roof_sec = None
-    if l2 and sectors and n_slabs > 1:
+    if l2 and sectors and n_slabs > 1 and not listed:
         # z-slab form: the gathers (pass A) and the REDs (pass B) run in separate launches,
         # each bound by its own access type's sector rate -> a two-pass ceiling
         g_sec, r_sec = tr["l2_sectors_read_per_launch"], tr["l2_sectors_red_per_launch"]
@@ -556,7 +564,7 @@ def main():
     # a RED one cycle per 32-byte sector (tools/request_probe.cu)
     roof_req = None
     clocks = clk.summary()
-    if sectors and tr.get("l2_requests_read_per_launch"):
+    if sectors and tr and tr.get("l2_requests_read_per_launch"):
         sm_hz = (clocks.get("sm_mhz") or peaks.get("sm_max_mhz") or 1965.0) * 1e6
         cyc = tr["l2_requests_read_per_launch"] + tr["l2_sectors_red_per_launch"]
         peak_req = torch.cuda.get_device_properties(dev).multi_processor_count * sm_hz
@@ -566,7 +574,7 @@ def main():
                     "what": "(gather requests + RED sectors) per launch (ncu, profiles/r02_traffic.json; summed over "
                             "a subset's launches in the z-slab form) / live duration, vs one request cycle per SM "
                             "clock (SMs x median SM clock under load)"}
-    hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0 * (2 * n_slabs if n_slabs > 1 else 1)) / proj_avg_s / 1e9,
+    hbm = {"bound": "hbm", "achieved": (ev_per_launch * 24.0 * ev_reads) / proj_avg_s / 1e9,
            "peak": peaks["hbm_gbs"],
            "unit": "GB/s", "peak_kind": peak_kind, "what": "event streaming of k_project (24 B/event)"}
     hbm["frac"] = hbm["achieved"] / hbm["peak"]

@@ -109,6 +109,7 @@ struct lmosem_ctx {
     int zfine_per = 2;         // fine slabs per coarse slab (LMOSEM_ZFINE)
     int zfused_mode = 5;       // k_project mode of the fine-window launches (LMOSEM_ZFUSED_MODE: 5 or 6)
     int zover = 2;             // fine windows overlap: stride = width / zover (LMOSEM_ZOVER)
+    int zwin = 0;              // fine window width in voxels (LMOSEM_ZWIN; 0: from zfine_per)
     int* zlist = nullptr;      // lists, zlist_cap indices each
     int* zcount = nullptr;     // their lengths (kZMaxLists)
     int64_t zlist_cap = 0;
@@ -768,7 +769,8 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         // pipe, MODE 5/6): width ~ 1/zfine_per of a coarse slab, stride width/zover, even planes
         std::vector<std::pair<int, int>> wins;
         const int na = ctx->dims[ctx->slab_axis];
-        const int W = 2 * std::max(1, na / (2 * K * ctx->zfine_per));
+        const int W = ctx->zwin > 0 ? std::min(na, 2 * ((ctx->zwin + 1) / 2))
+                                    : 2 * std::max(1, na / (2 * K * ctx->zfine_per));
         const int S = 2 * std::max(1, W / (2 * ctx->zover));
         if (ctx->zlist_mode == 2 && ctx->geom.tex_fb && W < na) {
             for (int lo = 0;; lo += S) {
@@ -1342,6 +1344,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (const char* e = std::getenv("LMOSEM_ZFINE")) ctx->zfine_per = std::max(1, std::min(8, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_ZFUSED_MODE")) ctx->zfused_mode = std::atoi(e) == 5 ? 5 : 6;
     if (const char* e = std::getenv("LMOSEM_ZOVER")) ctx->zover = std::max(1, std::min(4, std::atoi(e)));
+    if (const char* e = std::getenv("LMOSEM_ZWIN")) ctx->zwin = std::max(0, std::atoi(e));
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {

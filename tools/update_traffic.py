@@ -3,7 +3,9 @@
 --set full capture of that config's projection: DRAM bytes and L2 sectors (gathers, REDs)
 per launch of the fused kernel, or summed over the launches of one subset step (the C4
 z-slab form: 3 pass-A + 3 pass-B launches).
-Usage: update_traffic.py REPORT.ncu-rep SUMMARY_NAME [CONFIG] [LAUNCHES_PER_STEP]"""
+The listed z-slab form (C4: 3 pass-A + fine-window + 3 pass-B launches over k_zclass's lists)
+is marked form = "listed".
+Usage: update_traffic.py REPORT.ncu-rep SUMMARY_NAME [CONFIG] [LAUNCHES_PER_STEP] [FORM]"""
 import csv
 import io
 import json
@@ -15,7 +17,7 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 PATH = os.environ.get("LMOSEM_TRAFFIC_JSON") or os.path.join(ROOT, "profiles", "r02_traffic.json")
 
 
-def main(rep, summary, config="C2", per_step=1):
+def main(rep, summary, config="C2", per_step=1, form=None):
     raw = list(csv.reader(io.StringIO(subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"],
                                                      capture_output=True, text=True).stdout)))
     names, units, rows = raw[0], raw[1], raw[2:]
@@ -34,6 +36,7 @@ def main(rep, summary, config="C2", per_step=1):
     kernels = sorted({dict(zip(names, r)).get("Kernel Name", "?").split("(")[0] for r in rows})
     entry = {
         "kernel": ", ".join(kernels),
+        "form": form,
         "launches_per_step": per_step,
         "dram_bytes_read_per_launch": tot("dram__bytes_read.sum"),
         "dram_bytes_write_per_launch": tot("dram__bytes_write.sum"),
@@ -61,4 +64,4 @@ def main(rep, summary, config="C2", per_step=1):
 
 
 if __name__ == "__main__":
-    main(sys.argv[1], sys.argv[2], *(sys.argv[3:4]), *(int(x) for x in sys.argv[4:5]))
+    main(sys.argv[1], sys.argv[2], *(sys.argv[3:4]), *(int(x) for x in sys.argv[4:5]), *(sys.argv[5:6]))
