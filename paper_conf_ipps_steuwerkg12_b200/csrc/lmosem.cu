@@ -764,7 +764,7 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         CKA(cudaMalloc(&ctx->fp_acc, sizeof(float) * n));
         ctx->fp_cap = n;
     }
-    if (ctx->zlist_mode > 0 && n <= INT32_MAX) {
+    if (ctx->zlist_mode > 0 && n <= INT32_MAX && K <= lmk::kZMaxBits) {
         // fine windows along the slab axis (the fused launches gather through the texture
         // pipe, MODE 5/6): width ~ 1/zfine_per of a coarse slab, stride width/zover, even planes
         std::vector<std::pair<int, int>> wins;

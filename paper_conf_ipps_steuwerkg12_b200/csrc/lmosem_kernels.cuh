@@ -807,26 +807,28 @@ __device__ __forceinline__ unsigned zclass_bits(const float ev[6], const GridGeo
     return bits;
 }
 
-// One CTA per chunk of kZChunk consecutive events (grid-stride): the appends are counted per
-// warp in shared memory, then one global atomic per list and chunk reserves the chunk's
-// range (a global atomic per warp and list serialised on the K + Kf counters: 0.6-1.5 ms
-// per C4 subset). Within a list the events keep chunk order, within a chunk warp order.
-constexpr int kZThreads = 256, kZPer = 8, kZChunk = kZThreads * kZPer;
+// One CTA per chunk of kZChunk consecutive events (grid-stride): each event takes its slot in
+// each of its (<= kZMaxBits) lists with a shared-memory atomic, then one global atomic per
+// list and chunk reserves the chunk's range. (A global atomic per warp and list serialised on
+// the list counters: 0.6-1.5 ms per C4 subset; warp ballots per list: 0.44 ms.) Within a
+// list, events keep chunk order.
+#ifndef LMK_ZPER
+#define LMK_ZPER 4  // events per thread and chunk in k_zclass (A/B: 1 / 2 / 4 / 8 / 16: 161 / 137 / 138 / 194 / 358 us at C4)
+#endif
+constexpr int kZThreads = 256, kZPer = LMK_ZPER, kZChunk = kZThreads * kZPer;
+constexpr int kZMaxBits = 4;  // lists per event: one window, or <= 4 coarse slabs (host: K <= 4)
 __global__ void __launch_bounds__(kZThreads) k_zclass(const float* __restrict__ events, int64_t n, GridGeom g,
                                                       ZClass zc, int* __restrict__ lists, int64_t cap,
                                                       int* __restrict__ counts) {
     pdl_wait();
     pdl_trigger();
     __shared__ int s_cnt[kZMaxLists], s_base[kZMaxLists];
-    __shared__ int s_woff[kZThreads / 32][kZPer][kZMaxLists];
-    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-    const unsigned lt = (1u << lane) - 1u;
     const int nl = zc.K + zc.Kf;
     for (int64_t c0 = (int64_t)blockIdx.x * kZChunk; c0 < n; c0 += (int64_t)gridDim.x * kZChunk) {
         if ((int)threadIdx.x < nl) s_cnt[threadIdx.x] = 0;
         __syncthreads();
         unsigned bits[kZPer];
-        // all kZPer events' loads in flight before the float64 clips
+        // all kZPer events' loads in flight before the clips
         float ev[kZPer][6];
 #pragma unroll
         for (int p = 0; p < kZPer; ++p) {
@@ -836,14 +838,14 @@ __global__ void __launch_bounds__(kZThreads) k_zclass(const float* __restrict__ 
 #pragma unroll
         for (int p = 0; p < kZPer; ++p)
             bits[p] = c0 + p * kZThreads + threadIdx.x < n ? zclass_bits(ev[p], g, zc) : 0u;
+        int off[kZPer][kZMaxBits];
 #pragma unroll
         for (int p = 0; p < kZPer; ++p) {
-            unsigned any = __reduce_or_sync(0xffffffffu, bits[p]);
-            while (any) {
-                const int l = __ffs(any) - 1;
-                any &= any - 1;
-                const unsigned mask = __ballot_sync(0xffffffffu, (bits[p] >> l) & 1u);
-                if (lane == 0) s_woff[w][p][l] = atomicAdd(&s_cnt[l], __popc(mask));
+            unsigned b = bits[p];
+#pragma unroll
+            for (int q = 0; q < kZMaxBits; ++q) {
+                if (b) off[p][q] = atomicAdd(&s_cnt[__ffs(b) - 1], 1);
+                b &= b - 1;
             }
         }
         __syncthreads();
@@ -851,18 +853,18 @@ __global__ void __launch_bounds__(kZThreads) k_zclass(const float* __restrict__ 
         __syncthreads();
 #pragma unroll
         for (int p = 0; p < kZPer; ++p) {
-            unsigned any = __reduce_or_sync(0xffffffffu, bits[p]);
-            while (any) {
-                const int l = __ffs(any) - 1;
-                any &= any - 1;
-                const bool in = (bits[p] >> l) & 1u;
-                const unsigned mask = __ballot_sync(0xffffffffu, in);
-                if (in)
-                    lists[(int64_t)l * cap + s_base[l] + s_woff[w][p][l] + __popc(mask & lt)] =
-                        (int)(c0 + p * kZThreads + threadIdx.x);
+            unsigned b = bits[p];
+            const int e = (int)(c0 + p * kZThreads + threadIdx.x);
+#pragma unroll
+            for (int q = 0; q < kZMaxBits; ++q) {
+                if (b) {
+                    const int l = __ffs(b) - 1;
+                    lists[(int64_t)l * cap + s_base[l] + off[p][q]] = e;
+                }
+                b &= b - 1;
             }
         }
-        __syncthreads();  // s_cnt / s_woff are rewritten by the next chunk
+        __syncthreads();  // s_cnt / s_base are rewritten by the next chunk
     }
 }
 
