@@ -108,8 +108,9 @@ struct lmosem_ctx {
                                     // 2: + fused launches over fine slabs (LMOSEM_ZLIST)
     int zfine_per = 2;         // fine slabs per coarse slab (LMOSEM_ZFINE)
     int zfused_mode = 5;       // k_project mode of the fine-window launches (LMOSEM_ZFUSED_MODE: 5 or 6)
-    int zover = 2;             // fine windows overlap: stride = width / zover (LMOSEM_ZOVER)
+    int zover = 4;             // fine windows overlap: stride = width / zover (LMOSEM_ZOVER)
     int zwin = 0;              // fine window width in voxels (LMOSEM_ZWIN; 0: from zfine_per)
+    int zmerge = 1;            // the windows of a coarse slab in one launch (LMOSEM_ZMERGE)
     int* zlist = nullptr;      // lists, zlist_cap indices each
     int* zcount = nullptr;     // their lengths (kZMaxLists)
     int64_t zlist_cap = 0;
@@ -612,15 +613,16 @@ lmosem_status proj_occupancy(lmosem_ctx* ctx, int mode, size_t smem, int* blocks
     return LMOSEM_OK;
 }
 
-// list != nullptr (MODEs 2, 3, 5, 6): the launch runs over the events list[0 .. *list_n),
-// list_n <= n (on the device; n sizes the grid and the claims)
+// la != nullptr (MODEs 2, 3, 5, 6): the launch runs over the listed events of *la (their
+// number, <= n, is on the device; n sizes the grid)
 lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n, float* fp, const lmk::GridGeom& g,
-                          const int* list = nullptr, const int* list_n = nullptr) {
+                          const lmk::ListArg* la = nullptr) {
+    const bool list = la != nullptr;
     const int cap = launch_cap(mode, g);
     const int threads = lmk::proj_threads_of(mode);
     const size_t sm = (threads / 32) * (sizeof(int2) * (size_t)cap + lmk::lor_bytes_per_warp(mode));
     int per_sm = 1;
-    lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm, list != nullptr);
+    lmosem_status s = proj_occupancy(ctx, mode, sm, &per_sm, list);
     if (s) return s;
     const int64_t wpb = threads / 32;
     const int64_t resident = (int64_t)ctx->num_sms * per_sm * wpb;
@@ -638,7 +640,7 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
     // gains from the smaller final claims of divisor 3; a rank's share at P >= 2 from 2
     const int gdiv = n >= (int64_t)LMOSEM_GUIDED_ROUNDS * 32 * resident ? LMOSEM_GUIDED_LARGE : LMOSEM_GUIDED_SMALL;
     void (*k)(const float*, int64_t, const float*, float*, float*, lmk::GridGeom, int, unsigned long long*, int, int,
-              const int*, const int*);
+              lmk::ListArg);
     if (list) switch (mode) {
         case 2: k = lmk::k_project<2, true>; break;
         case 3: k = lmk::k_project<3, true>; break;
@@ -653,8 +655,9 @@ lmosem_status launch_mode(lmosem_ctx* ctx, int mode, const float* evf, int64_t n
         case 5: k = lmk::k_project<5>; break;
         default: k = lmk::k_project<6>; break;
     }
-    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch, gdiv, list,
-                list_n));
+    const lmk::ListArg none{};
+    CK(launch_k(ctx, k, grid, threads, sm, evf, n, (const float*)ctx->fb, ctx->c, fp, g, cap, work, batch, gdiv,
+                list ? *la : none));
     return LMOSEM_OK;
 }
 
@@ -714,27 +717,51 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
                 ctx->zcount));
     // the first listed launch reads the lists before griddepcontrol.wait: a plain launch
     ctx->after_kernel = false;
-    const int* X = ctx->zlist;
     lmosem_status s;
-    for (int k = 0; k < K; ++k)
-        if ((s = launch_mode(ctx, 2, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), X + (size_t)k * ctx->zlist_cap,
-                             ctx->zcount + k)))
-            return s;
+    auto one_list = [&](int l) {
+        lmk::ListArg la{};
+        la.lists = ctx->zlist;
+        la.counts = ctx->zcount;
+        la.cap = ctx->zlist_cap;
+        la.first = l;
+        la.nseg = 1;
+        la.axis = zc.axis;
+        return la;
+    };
+    for (int k = 0; k < K; ++k) {
+        const lmk::ListArg la = one_list(k);
+        if ((s = launch_mode(ctx, 2, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), &la))) return s;
+    }
     const int fused = ctx->zfused_mode;
     for (int k = 0; k < K; ++k) {
-        for (int j = 0; j < Kf; ++j) {
+        // the windows centred in slab k, in order, as one launch (up to kMaxSeg per launch, or
+        // one per window with LMOSEM_ZMERGE=0): their lists are claimed in sequence, so the
+        // LORs in flight stay within about one window
+        int j = 0;
+        while (j < Kf) {
             const int mid = (zc.wlo[j] + zc.whi[j]) / 2;
-            if (mid < zc.cb[k] || mid >= zc.cb[k + 1]) continue;  // window j runs before pass B of its centre's slab
-            lmk::GridGeom gj = ctx->geom;
+            if (mid < zc.cb[k] || mid >= zc.cb[k + 1]) {
+                ++j;
+                continue;
+            }
+            lmk::ListArg la = one_list(K + j);
+            la.box = 1;
+            la.nseg = 0;
+            lmk::GridGeom gj = ctx->geom;  // the window box (equal widths: sizes the path buffers)
             gj.clo[zc.axis] = zc.wlo[j];
             gj.chi[zc.axis] = zc.whi[j];
-            if ((s = launch_mode(ctx, fused, evf, n, nullptr, gj, X + (size_t)(K + j) * ctx->zlist_cap,
-                                 ctx->zcount + K + j)))
-                return s;
+            const int per = ctx->zmerge ? lmk::kMaxSeg : 1;
+            for (; j < Kf && la.nseg < per; ++j) {
+                const int mj = (zc.wlo[j] + zc.whi[j]) / 2;
+                if (mj < zc.cb[k] || mj >= zc.cb[k + 1]) break;
+                la.lo[la.nseg] = zc.wlo[j];
+                la.hi[la.nseg] = zc.whi[j];
+                la.nseg++;
+            }
+            if ((s = launch_mode(ctx, fused, evf, n, nullptr, gj, &la))) return s;
         }
-        if ((s = launch_mode(ctx, 3, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), X + (size_t)k * ctx->zlist_cap,
-                             ctx->zcount + k)))
-            return s;
+        const lmk::ListArg lb = one_list(k);
+        if ((s = launch_mode(ctx, 3, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), &lb))) return s;
     }
     return LMOSEM_OK;
 }
@@ -1345,6 +1372,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (const char* e = std::getenv("LMOSEM_ZFUSED_MODE")) ctx->zfused_mode = std::atoi(e) == 5 ? 5 : 6;
     if (const char* e = std::getenv("LMOSEM_ZOVER")) ctx->zover = std::max(1, std::min(4, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_ZWIN")) ctx->zwin = std::max(0, std::atoi(e));
+    if (const char* e = std::getenv("LMOSEM_ZMERGE")) ctx->zmerge = e[0] != '0';
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {
@@ -1363,17 +1391,25 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     // a larger one (each launch passes its own size).
     {
         const int smax = (int)prop.sharedMemPerBlockOptin;
-        cuda(cudaFuncSetAttribute(lmk::k_project<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<5>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<6>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<2, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<3, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<5, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
-        cuda(cudaFuncSetAttribute(lmk::k_project<6, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smax), "smem attr");
+        // dynamic shared memory up to the opt-in limit less the kernel's static shared memory
+        // (the listed variants keep their segment table there)
+        auto smem_max = [&](auto kern) {
+            cudaFuncAttributes fa{};
+            cuda(cudaFuncGetAttributes(&fa, kern), "func attr");
+            cuda(cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                      smax - (int)fa.sharedSizeBytes), "smem attr");
+        };
+        smem_max(lmk::k_project<0>);
+        smem_max(lmk::k_project<1>);
+        smem_max(lmk::k_project<2>);
+        smem_max(lmk::k_project<3>);
+        smem_max(lmk::k_project<4>);
+        smem_max(lmk::k_project<5>);
+        smem_max(lmk::k_project<6>);
+        smem_max(lmk::k_project<2, true>);
+        smem_max(lmk::k_project<3, true>);
+        smem_max(lmk::k_project<5, true>);
+        smem_max(lmk::k_project<6, true>);
     }
     cuda(cudaStreamCreateWithFlags(&ctx->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     cuda(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking), "cudaStreamCreate");

@@ -88,7 +88,9 @@ __device__ __forceinline__ T sel3(const T (&v)[3], int i) {
 // float64. There the clip (volume entry and exit, segment ends, slab-pass boundaries) meets
 // the plane crossings, and a piece between a clip and a crossing must not be the difference
 // of two rounded floats (a 3.7e-4-slab piece carried 1.5e-4 relative error that way).
-__device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const GridGeom& g, Lor& L, float clip[6]) {
+// clo/chi: the launch's clip box (g.clo/g.chi, or a fused window's box in a listed launch).
+__device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const GridGeom& g, const int (&clo)[3],
+                                          const int (&chi)[3], Lor& L, float clip[6]) {
     double p1[3], d[3], u1[3], D[3], rD[3];
     bool ok = true;
 #pragma unroll
@@ -111,7 +113,7 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     double amin = 0.0, amax = 1.0;
 #pragma unroll
     for (int k = 0; k < 3; ++k) {
-        const double lo = (double)g.clo[k], hi = (double)g.chi[k];
+        const double lo = (double)clo[k], hi = (double)chi[k];
         rD[k] = 0.0;
         if (D[k] != 0.0) {
             const double r = 1.0 / D[k];
@@ -132,8 +134,8 @@ __device__ __forceinline__ bool lor_setup(const float* __restrict__ ev, const Gr
     const double Db = sel3(D, b), Dc = sel3(D, c), u1b = sel3(u1, b), u1c = sel3(u1, c);
     double ua_in = u1a + amin * Da, ua_out = u1a + amax * Da;
     if (Da < 0.0) { double t = ua_in; ua_in = ua_out; ua_out = t; }
-    int i0 = max((int)floor(ua_in), sel3(g.clo, a));
-    int il = min((int)ceil(ua_out) - 1, sel3(g.chi, a) - 1);
+    int i0 = max((int)floor(ua_in), sel3(clo, a));
+    int il = min((int)ceil(ua_out) - 1, sel3(chi, a) - 1);
     if (il < i0) return false;
     const double rDa = sel3(rD, a);  // 1 / Da from the clip (Da != 0: the dominant axis)
     const double sb = Db * rDa, sc = Dc * rDa;
@@ -496,15 +498,26 @@ __host__ __device__ constexpr int proj_threads_of(int mode) {
 //         claims per warp).
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
-// LIST (MODEs 2, 3, 5, 6; the listed z-slab form): the launch runs over the events
-// list[0 .. *list_n) (indices into `events` and `fp`, written by k_zclass) instead of [0, n).
+// A listed launch (the listed z-slab form) runs over the concatenation of lists
+// first .. first + nseg - 1 of k_zclass (list l: lists + l * cap, length counts[l]; indices into
+// `events` and `fp`), in order. box = 1 (the fused windows): an event of segment s is clipped
+// to [lo[s], hi[s]) along `axis` instead of the launch's box.
+constexpr int kMaxSeg = 8;
+struct ListArg {
+    const int* lists;
+    const int* counts;
+    long long cap;
+    int first, nseg, axis, box;
+    int lo[kMaxSeg], hi[kMaxSeg];
+};
+
+// LIST (MODEs 2, 3, 5, 6): the launch runs over the listed events of `la` instead of [0, n).
 template <int MODE, bool LIST = false>
 __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>()) k_project(const float* __restrict__ events, int64_t n,
                                                              const float* __restrict__ fb, float* __restrict__ cb,
                                                              float* __restrict__ fp, GridGeom g, int cap,
                                                              unsigned long long* __restrict__ work, int batch,
-                                                             int gdiv, const int* __restrict__ list,
-                                                             const int* __restrict__ list_n) {
+                                                             int gdiv, ListArg la) {
     constexpr bool kGather = MODE <= 2 || MODE >= 5;  // forward projection in this launch
     constexpr bool kScatter = MODE == 0 || MODE >= 3;  // back-projection
     constexpr bool kTex = MODE >= 5;  // gathers of f through the texture path
@@ -532,8 +545,22 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     // the grid for all events; the claim sizes follow the list's length (lmosem.cu
     // launch_mode's rule with its defaults: first claims 32 halved while a warp would get
     // fewer than 4, >= 4; guided divisor 3 from 6 rounds of 32-event claims, else 2)
+    // ends of the segments in the concatenation, and their clip planes (static indices here:
+    // a dynamic index into the parameter array would copy it to the stack)
+    __shared__ int s_segend[LIST ? kMaxSeg : 1], s_seglo[LIST ? kMaxSeg : 1], s_seghi[LIST ? kMaxSeg : 1];
     if (LIST) {
-        n = (int64_t)*list_n;
+        int acc = 0;
+#pragma unroll
+        for (int q = 0; q < kMaxSeg; ++q) {
+            if (q < la.nseg) acc += __ldg(la.counts + la.first + q);
+            if (threadIdx.x == 0) {
+                s_segend[q] = acc;
+                s_seglo[q] = la.lo[q];
+                s_seghi[q] = la.hi[q];
+            }
+        }
+        __syncthreads();
+        n = (int64_t)acc;
         take = 32;
         while (take > 4 && n < (int64_t)take * warps_in_grid * 4) take >>= 1;
         batch = take;
@@ -569,8 +596,17 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         }
         const int64_t idx = base + lane;
         const bool mine_ev = lane < take && idx < n;
-        // the event (and fp slot) of this lane: idx, or the idx-th listed event
-        const int64_t eidx = LIST ? (mine_ev ? (int64_t)__ldg(list + idx) : 0) : idx;
+        // the event (and fp slot) of this lane: idx, or the idx-th listed event (segment sg)
+        int64_t eidx = idx;
+        int sg = 0;
+        if (LIST) {
+            eidx = 0;
+            if (mine_ev) {
+                int lo_i = 0;
+                while (sg < la.nseg - 1 && idx >= s_segend[sg]) lo_i = s_segend[sg++];
+                eidx = (int64_t)__ldg(la.lists + (int64_t)(la.first + sg) * la.cap + (idx - lo_i));
+            }
+        }
         // event tile staging: the claimed events (24 B each, contiguous) are loaded with
         // coalesced 16-byte vector loads into the head of the warp's path buffer (idle at
         // this point), then each lane reads its record from shared memory
@@ -601,7 +637,14 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 load_event(events, eidx, ev);
             }
             float clip[6];
-            ok = lor_setup(ev, g, mine, clip);
+            int clo[3], chi[3];
+#pragma unroll
+            for (int k = 0; k < 3; ++k) {
+                const bool w = LIST && la.box && k == la.axis;
+                clo[k] = w ? s_seglo[sg] : g.clo[k];
+                chi[k] = w ? s_seghi[sg] : g.chi[k];
+            }
+            ok = lor_setup(ev, g, clo, chi, mine, clip);
             if (ok && kLorSmem) {
                 lor_store(lor_w + kRec * (unsigned)lane, mine, clip);
             } else if (ok) {
