@@ -53,15 +53,17 @@ def rel_l2(got, ref):
     return v
 
 
-def run_world(pkg, P, cfg, s, combine, call, f0=None):
+def run_world(pkg, P, cfg, s, combine, call, f0=None, slabs=0):
     """Creates P loopback ranks (own stream each), runs call(rec, f) on every rank from its
-    own thread, and returns the P f images (float64 numpy) plus each rank's stats."""
+    own thread, and returns the P f images (float64 numpy) plus each rank's stats. slabs > 0
+    forces the z-slab form (the listed one by default) on every rank."""
     group = pkg.Loopback(P)
     recs, fs = [], []
     f0 = np.ones(cfg.n_voxels, np.float32) if f0 is None else f0.astype(np.float32)
     for r in range(P):
         rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s), stream=torch.cuda.Stream(), loopback=(group, r))
         rec.set_combine(combine)
+        rec.set_slabs(slabs)
         assert rec.combine == combine and rec.world == P and rec.rank == r
         recs.append(rec)
         fs.append(dev(f0))
@@ -131,6 +133,26 @@ def test_loopback_c1_subset_and_reconstruction(pkg, P, combine):
     off = np.arange(cfg.n_subsets + 1) * cfg.n_events
     d_ev = dev(ev)
     got2, _ = run_world(pkg, P, cfg, s, combine, lambda rec, f: rec.reconstruct(d_ev, off, 2, f))
+    ref2 = cached(("C1", "recon2"), lambda: oracle.reconstruct(g, ev, off, 2, s, np.ones(cfg.n_voxels)))
+    assert rel_l2(got2, ref2) <= REL_L2_RECON
+
+
+@pytest.mark.parametrize("combine", COMBINES)
+@pytest.mark.parametrize("P,slabs", [(2, 2), (3, 3), (8, 2)])
+def test_loopback_listed_zslab_form(pkg, P, slabs, combine):
+    """The out-of-L2 step 1 (listed z-slab form: per-rank k_zclass lists of the rank's block,
+    passes A/B and fused window launches) under P ranks and every combine: one C1 subset and
+    2 subsets x 2 iterations against the oracle, replicas bitwise equal."""
+    cfg, ev, s = c1()
+    g = oracle.geom(cfg.dims, cfg.voxel_mm)
+    ev0 = ev[:cfg.n_events]
+    d_ev0 = dev(ev0)
+    got, _ = run_world(pkg, P, cfg, s, combine, lambda rec, f: rec.subset_step(d_ev0, f), slabs=slabs)
+    ref = cached(("C1", "subset"), lambda: oracle.subset_step(g, ev0, s, np.ones(cfg.n_voxels)))
+    assert maxrel(got, ref) <= MAXREL_SUBSET
+    off = np.arange(cfg.n_subsets + 1) * cfg.n_events
+    d_ev = dev(ev)
+    got2, _ = run_world(pkg, P, cfg, s, combine, lambda rec, f: rec.reconstruct(d_ev, off, 2, f), slabs=slabs)
     ref2 = cached(("C1", "recon2"), lambda: oracle.reconstruct(g, ev, off, 2, s, np.ones(cfg.n_voxels)))
     assert rel_l2(got2, ref2) <= REL_L2_RECON
 
