@@ -84,6 +84,20 @@ MUTANTS = [
      "bx + 1 < (unsigned)it.rhi[0]", False),
     ("fused combine: local c not re-zeroed", K, "            C[2 * b] = z;\n            C[2 * b + 1] = z;\n", "", False),
     ("fused combine: second brick of a pair not stored", K, "            team.store_f(ob, nb0, nb1);\n", "", False),
+    # the listed z-slab form (round 2: caught by tests/test_zlist_gpu.py and the loopback test)
+    ("listed: window membership without its margin", K, "if (zl >= lo + m && zh <= lo + zc.ww - m) return",
+     "if (zl >= lo - m && zh <= lo + zc.ww + m) return", False),
+    ("listed: coarse membership shrunk by the margin", K,
+     "if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) bits |= 1u << k;",
+     "if (zh > (float)zc.cb[k] + m && zl < (float)zc.cb[k + 1] - m) bits |= 1u << k;", False),
+    ("listed: window LORs also in the coarse lists", K, "return 1u << (zc.K + j);", "return (1u << (zc.K + j)) | all;",
+     False),
+    ("listed: list slots without the per-event offset", K, "lists[(int64_t)l * cap + s_base[l] + off[p][q]] = e;",
+     "lists[(int64_t)l * cap + s_base[l]] = e;", False),
+    ("listed: segment lookup off by one", K, "while (sg < la.nseg - 1 && idx >= s_segend[sg])",
+     "while (sg < la.nseg - 1 && idx > s_segend[sg])", False),
+    ("listed: window box not applied per event", K, "const bool w = LIST && la.box && k == la.axis;",
+     "const bool w = false;", False),
 ]
 # Not listed: equivalent mutants. Dropping the 2^-40 offset of the mirrored frame changes
 # only exactly integral up-moving positions, where "voxel m - 1 with a crossing at d = 0"
@@ -93,7 +107,7 @@ MUTANTS = [
 # covered by the gloo tests and the emulated-rank combine test). The z-slab pass B setup
 # test `ok && fp_known > 0` only saves work: the back-projection's own fp > 0 guard skips
 # the same events (measured: the mutant passes every parity test, as expected).
-TESTS = ("loopback_c1 or loopback_c2 or loopback_ragged or golden or degenerate or axis_parallel or c1_ or zslab_passes_match_oracle_c1 or odd_extents or "
+TESTS = ("listed or loopback_c1 or loopback_c2 or loopback_ragged or golden or degenerate or axis_parallel or c1_ or zslab_passes_match_oracle_c1 or odd_extents or "
          "lors_in_voxel_faces or one_subset_paper_shaped or programmatic or nccl_combine_single_rank or "
          "combine_modes_single_rank or zero_forward_projection or lsu_and_texture")
 
@@ -132,7 +146,8 @@ def run(only=None):
             continue
         env = dict(os.environ, LMOSEM_LIB=os.path.join(OUT, f"liblmosem_m{i}.so"))
         out = subprocess.run([sys.executable, "-m", "pytest", os.path.join(ROOT, "tests", "test_parity_gpu.py"),
-                              os.path.join(ROOT, "tests", "test_loopback_gpu.py"), "-x",
+                              os.path.join(ROOT, "tests", "test_loopback_gpu.py"),
+                              os.path.join(ROOT, "tests", "test_zlist_gpu.py"), "-x",
                               "-q", "-p", "no:cacheprovider", "-k", TESTS], capture_output=True, text=True, cwd=ROOT,
                              env=env, timeout=900)
         tail = [ln for ln in out.stdout.splitlines() if ln.startswith("FAILED") or " passed" in ln or " failed" in ln]
