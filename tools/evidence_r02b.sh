@@ -2,7 +2,7 @@
 # Round 2 (listed z-slab form): GPU suite, C4 traffic capture of the listed launches (updates
 # profiles/r02_traffic.json C4 on the box copy; copied back by hand), ncu --set full of a
 # pass-B and a fine-window launch, bench lines C2/C4/C5 + reference, smoke, launch list.
-O=gpurun_out/ev3
+O=gpurun_out/${EV_OUT:-ev3}
 mkdir -p $O
 python -c "import __graft_entry__ as g; g.build()" > $O/build.txt 2>&1 || { echo BUILD FAILED; tail -5 $O/build.txt; exit 1; }
 (echo "# pytest -m gpu -v -s (one B200): per-test parity errors vs the float64 oracle"; timeout 1500 python -m pytest tests -m gpu -v -s -p no:cacheprovider 2>&1 | grep -E "parity|watchdog|PASSED|FAILED|passed|failed|Error") > $O/parity.txt
@@ -14,7 +14,7 @@ LMOSEM_TRAFFIC_JSON=$O/r02_traffic.json python tools/update_traffic.py $O/c4_lis
 ncu -i $O/c4_listed_traffic.ncu-rep --page raw --csv > $O/c4_listed_traffic.csv 2>/dev/null
 cp $O/r02_traffic.json profiles/r02_traffic.json
 ncu --set full --clock-control none --import-source on -k regex:k_project -s 35 -c 1 -o $O/k_project_C4_passB python bench.py --config C4 --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
-ncu --set full --clock-control none --import-source on -k regex:k_project -s 30 -c 1 -o $O/k_project_C4_window python bench.py --config C4 --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
+ncu --set full --clock-control none --import-source on -k regex:k_project -s 32 -c 1 -o $O/k_project_C4_window python bench.py --config C4 --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > /dev/null 2>&1
 for r in k_project_C4_passB k_project_C4_window; do python tools/ncu_summary.py $O/$r.ncu-rep > $O/${r}_summary.txt 2>&1; done
 python bench.py > $O/bench_C2.json 2> $O/bench_C2.err
 python bench.py --config C5 > $O/bench_C5.json 2> /dev/null
