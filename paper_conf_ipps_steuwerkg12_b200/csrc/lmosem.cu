@@ -798,12 +798,16 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         const int na = ctx->dims[ctx->slab_axis];
         const int W = ctx->zwin > 0 ? std::min(na, 2 * ((ctx->zwin + 1) / 2))
                                     : 2 * std::max(1, na / (2 * K * ctx->zfine_per));
-        const int S = 2 * std::max(1, W / (2 * ctx->zover));
         if (ctx->zlist_mode == 2 && ctx->geom.tex_fb && W < na) {
-            for (int lo = 0;; lo += S) {
-                const int l = std::min(lo, na - W);
-                wins.push_back({l, l + W});
-                if (l + W >= na) break;
+            // the stride grows (fewer, less overlapping windows) until the lists fit kZMaxLists
+            for (int S = 2 * std::max(1, W / (2 * ctx->zover));; S += 2) {
+                wins.clear();
+                for (int lo = 0;; lo += S) {
+                    const int l = std::min(lo, na - W);
+                    wins.push_back({l, l + W});
+                    if (l + W >= na) break;
+                }
+                if (K + (int)wins.size() <= lmk::kZMaxLists) break;
             }
         }
         if (K + (int)wins.size() <= lmk::kZMaxLists) return launch_project_listed(ctx, evf, n, K, wins);

@@ -59,7 +59,8 @@ def subset_case(name):
 #  ZMERGE: the windows of a coarse slab in one launch)
 FORMS = [("0", "2", "6", "1", "0", "1"), ("1", "2", "6", "1", "0", "1"), ("2", "2", "6", "1", "0", "1"),
          ("2", "1", "6", "1", "0", "1"), ("2", "3", "5", "1", "0", "1"), ("2", "2", "6", "2", "0", "1"),
-         ("2", "3", "6", "3", "0", "1"), ("2", "2", "5", "2", "0", "0"), ("2", "2", "5", "2", "20", "1")]
+         ("2", "3", "6", "3", "0", "1"), ("2", "2", "5", "2", "0", "0"), ("2", "2", "5", "2", "20", "1"),
+         ("2", "2", "5", "4", "8", "1")]
 
 
 @pytest.mark.parametrize("zlist,zfine,zmode,zover,zwin,zmerge", FORMS)
@@ -67,7 +68,8 @@ FORMS = [("0", "2", "6", "1", "0", "1"), ("1", "2", "6", "1", "0", "1"), ("2", "
 def test_listed_zslab_subset_matches_oracle(pkg, monkeypatch, zlist, zfine, zmode, zover, zwin, zmerge, name,
                                             slabs):
     """ZWIN=20 at C2 with 3 slabs: 27 windows, 9 centred in a coarse slab -> two merged launches
-    (kMaxSeg = 8); C1 with 5 slabs runs the unlisted form (listed needs <= 4 coarse slabs)."""
+    (kMaxSeg = 8); ZWIN=8 at stride 2 would need > 32 lists at C2: the stride grows until they
+    fit; C1 with 5 slabs runs the unlisted form (listed needs <= 4 coarse slabs)."""
     for k, v in (("ZLIST", zlist), ("ZFINE", zfine), ("ZFUSED_MODE", zmode), ("ZOVER", zover), ("ZWIN", zwin),
                  ("ZMERGE", zmerge)):
         monkeypatch.setenv("LMOSEM_" + k, v)
