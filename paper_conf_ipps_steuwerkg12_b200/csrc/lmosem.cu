@@ -111,6 +111,7 @@ struct lmosem_ctx {
     int zover = 4;             // fine windows overlap: stride = width / zover (LMOSEM_ZOVER)
     int zwin = 0;              // fine window width in voxels (LMOSEM_ZWIN; 0: from zfine_per)
     int zmerge = 1;            // the windows of a coarse slab in one launch (LMOSEM_ZMERGE)
+    int zmed = 3;              // medium windows: stride = coarse width / zmed (LMOSEM_ZMED; 0: none)
     int* zlist = nullptr;      // lists, zlist_cap indices each
     int* zcount = nullptr;     // their lengths (kZMaxLists)
     int64_t zlist_cap = 0;
@@ -677,9 +678,10 @@ lmk::GridGeom slab_geom(const lmosem_ctx* ctx, int k, int K) {
 // coarse slab (fp of the X LORs complete), then per coarse slab k the fused launches of its
 // fine slabs and pass B of X_k, so c's slab k stays L2-resident across them.
 lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n, int K,
-                                   const std::vector<std::pair<int, int>>& wins) {
-    const int Kf = (int)wins.size();
-    const int nl = K + Kf;
+                                   const std::vector<std::pair<int, int>>& wins,
+                                   const std::vector<std::pair<int, int>>& mwins) {
+    const int Kf = (int)wins.size(), Km = (int)mwins.size();
+    const int nl = K + Kf + Km;
     if (n > ctx->zlist_cap || nl > ctx->zlist_n) {
         if (ctx->zlist) CK(cudaFree(ctx->zlist));
         ctx->zlist = nullptr;
@@ -693,6 +695,7 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
     lmk::ZClass zc{};
     zc.K = K;
     zc.Kf = Kf;
+    zc.Km = Km;
     zc.axis = ctx->slab_axis;
     for (int k = 0; k < K; ++k) {
         const lmk::GridGeom gk = slab_geom(ctx, k, K);
@@ -703,11 +706,15 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
         zc.wlo[j] = wins[j].first;
         zc.whi[j] = wins[j].second;
     }
-    if (Kf > 0) {  // windows j * stride (the last one clamped to end at the axis' end), equal widths
-        zc.ws = Kf > 1 ? (float)wins[1].first : 1.0f;
-        zc.ww = (float)(wins[0].second - wins[0].first);
-        zc.wlast = (float)wins[Kf - 1].first;
-    }
+    // a window family: starts j * stride (the last one clamped to end at the axis' end), equal widths
+    auto family = [](const std::vector<std::pair<int, int>>& w, float& stride, float& width, float& last) {
+        if (w.empty()) return;
+        stride = w.size() > 1 ? (float)w[1].first : 1.0f;
+        width = (float)(w[0].second - w[0].first);
+        last = (float)w.back().first;
+    };
+    family(wins, zc.ws, zc.ww, zc.wlast);
+    family(mwins, zc.ms, zc.mw, zc.mlast);
     not_kernel(ctx);
     CK(cudaMemsetAsync(ctx->zcount, 0, sizeof(int) * lmk::kZMaxLists, ctx->stream));
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
@@ -718,20 +725,41 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
     // the first listed launch reads the lists before griddepcontrol.wait: a plain launch
     ctx->after_kernel = false;
     lmosem_status s;
-    auto one_list = [&](int l) {
-        lmk::ListArg la{};
-        la.lists = ctx->zlist;
-        la.counts = ctx->zcount;
-        la.cap = ctx->zlist_cap;
-        la.first = l;
-        la.nseg = 1;
-        la.axis = zc.axis;
-        return la;
+    auto in_slab = [&](const std::pair<int, int>& w, int k) {  // a window runs with the slab of its centre
+        const int mid = (w.first + w.second) / 2;
+        return mid >= zc.cb[k] && mid < zc.cb[k + 1];
     };
-    for (int k = 0; k < K; ++k) {
-        const lmk::ListArg la = one_list(k);
-        if ((s = launch_mode(ctx, 2, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), &la))) return s;
-    }
+    // passes A / B of region k: coarse slab k's list, then the medium windows centred in it
+    // (each event clipped to its own segment's box; the path buffers sized for the widest)
+    auto two_pass = [&](int mode, int k) -> lmosem_status {
+        struct Seg { int list, lo, hi; };
+        std::vector<Seg> segs{{k, zc.cb[k], zc.cb[k + 1]}};
+        for (int j = 0; j < Km; ++j)
+            if (in_slab(mwins[j], k)) segs.push_back({K + Kf + j, mwins[j].first, mwins[j].second});
+        for (size_t i = 0; i < segs.size(); i += lmk::kMaxSeg) {
+            lmk::ListArg la{};
+            la.lists = ctx->zlist;
+            la.counts = ctx->zcount;
+            la.cap = ctx->zlist_cap;
+            la.axis = zc.axis;
+            la.box = 1;
+            la.nseg = (int)std::min<size_t>(lmk::kMaxSeg, segs.size() - i);
+            int widest = 0;
+            for (int q = 0; q < la.nseg; ++q) {
+                la.list[q] = segs[i + q].list;
+                la.lo[q] = segs[i + q].lo;
+                la.hi[q] = segs[i + q].hi;
+                widest = std::max(widest, segs[i + q].hi - segs[i + q].lo);
+            }
+            lmk::GridGeom g = ctx->geom;  // only sizes the path buffers: the widest segment box
+            g.clo[zc.axis] = 0;
+            g.chi[zc.axis] = widest;
+            if ((s = launch_mode(ctx, mode, evf, n, ctx->fp_acc, g, &la))) return s;
+        }
+        return LMOSEM_OK;
+    };
+    for (int k = 0; k < K; ++k)
+        if ((s = two_pass(2, k))) return s;
     const int fused = ctx->zfused_mode;
     for (int k = 0; k < K; ++k) {
         // the windows centred in slab k, in order, as one launch (up to kMaxSeg per launch, or
@@ -739,29 +767,29 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
         // LORs in flight stay within about one window
         int j = 0;
         while (j < Kf) {
-            const int mid = (zc.wlo[j] + zc.whi[j]) / 2;
-            if (mid < zc.cb[k] || mid >= zc.cb[k + 1]) {
+            if (!in_slab(wins[j], k)) {
                 ++j;
                 continue;
             }
-            lmk::ListArg la = one_list(K + j);
+            lmk::ListArg la{};
+            la.lists = ctx->zlist;
+            la.counts = ctx->zcount;
+            la.cap = ctx->zlist_cap;
+            la.axis = zc.axis;
             la.box = 1;
-            la.nseg = 0;
             lmk::GridGeom gj = ctx->geom;  // the window box (equal widths: sizes the path buffers)
             gj.clo[zc.axis] = zc.wlo[j];
             gj.chi[zc.axis] = zc.whi[j];
             const int per = ctx->zmerge ? lmk::kMaxSeg : 1;
-            for (; j < Kf && la.nseg < per; ++j) {
-                const int mj = (zc.wlo[j] + zc.whi[j]) / 2;
-                if (mj < zc.cb[k] || mj >= zc.cb[k + 1]) break;
+            for (; j < Kf && la.nseg < per && in_slab(wins[j], k); ++j) {
+                la.list[la.nseg] = K + j;
                 la.lo[la.nseg] = zc.wlo[j];
                 la.hi[la.nseg] = zc.whi[j];
                 la.nseg++;
             }
             if ((s = launch_mode(ctx, fused, evf, n, nullptr, gj, &la))) return s;
         }
-        const lmk::ListArg lb = one_list(k);
-        if ((s = launch_mode(ctx, 3, evf, n, ctx->fp_acc, slab_geom(ctx, k, K), &lb))) return s;
+        if ((s = two_pass(3, k))) return s;
     }
     return LMOSEM_OK;
 }
@@ -794,23 +822,39 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
     if (ctx->zlist_mode > 0 && n <= INT32_MAX && K <= lmk::kZMaxBits) {
         // fine windows along the slab axis (the fused launches gather through the texture
         // pipe, MODE 5/6): width ~ 1/zfine_per of a coarse slab, stride width/zover, even planes
-        std::vector<std::pair<int, int>> wins;
+        std::vector<std::pair<int, int>> wins, mwins;
         const int na = ctx->dims[ctx->slab_axis];
+        // windows [l, l + width) every `stride` voxels (the last one ends at the axis' end)
+        auto make = [na](std::vector<std::pair<int, int>>& w, int width, int stride) {
+            w.clear();
+            for (int lo = 0;; lo += stride) {
+                const int l = std::min(lo, na - width);
+                w.push_back({l, l + width});
+                if (l + width >= na) break;
+            }
+        };
         const int W = ctx->zwin > 0 ? std::min(na, 2 * ((ctx->zwin + 1) / 2))
                                     : 2 * std::max(1, na / (2 * K * ctx->zfine_per));
         if (ctx->zlist_mode == 2 && ctx->geom.tex_fb && W < na) {
             // the stride grows (fewer, less overlapping windows) until the lists fit kZMaxLists
             for (int S = 2 * std::max(1, W / (2 * ctx->zover));; S += 2) {
-                wins.clear();
-                for (int lo = 0;; lo += S) {
-                    const int l = std::min(lo, na - W);
-                    wins.push_back({l, l + W});
-                    if (l + W >= na) break;
-                }
-                if (K + (int)wins.size() <= lmk::kZMaxLists) break;
+                make(wins, W, S);
+                if (K + (int)wins.size() <= lmk::kZMaxLists || S >= na) break;
             }
         }
-        if (K + (int)wins.size() <= lmk::kZMaxLists) return launch_project_listed(ctx, evf, n, K, wins);
+        // medium windows (LMOSEM_ZMED > 0): as wide as a coarse slab, stride width / zmed, for
+        // the LORs that leave every fine window but fit one coarse-slab width: passes A and B
+        // over that one window instead of over each coarse slab they meet (with what is left
+        // of the list budget; none if it does not fit)
+        const int Wm = 2 * ((max_slab_extent(na, K) + 1) / 2);
+        if (ctx->zmed > 0 && K > 1 && Wm < na) {
+            for (int S = 2 * std::max(1, Wm / (2 * ctx->zmed));; S += 2) {
+                make(mwins, Wm, S);
+                if (K + (int)wins.size() + (int)mwins.size() <= lmk::kZMaxLists || S >= na) break;  // >= 2 windows remain
+            }
+            if (K + (int)wins.size() + (int)mwins.size() > lmk::kZMaxLists) mwins.clear();
+        }
+        if (K + (int)wins.size() <= lmk::kZMaxLists) return launch_project_listed(ctx, evf, n, K, wins, mwins);
     }
     not_kernel(ctx);
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
@@ -1377,6 +1421,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (const char* e = std::getenv("LMOSEM_ZOVER")) ctx->zover = std::max(1, std::min(4, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_ZWIN")) ctx->zwin = std::max(0, std::atoi(e));
     if (const char* e = std::getenv("LMOSEM_ZMERGE")) ctx->zmerge = e[0] != '0';
+    if (const char* e = std::getenv("LMOSEM_ZMED")) ctx->zmed = std::max(0, std::min(8, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {

@@ -498,17 +498,17 @@ __host__ __device__ constexpr int proj_threads_of(int mode) {
 //         claims per warp).
 // MODEs 2/3 are the out-of-L2 strategy: each pass touches only one
 // L2-sized slab of the image.
-// A listed launch (the listed z-slab form) runs over the concatenation of lists
-// first .. first + nseg - 1 of k_zclass (list l: lists + l * cap, length counts[l]; indices into
-// `events` and `fp`), in order. box = 1 (the fused windows): an event of segment s is clipped
-// to [lo[s], hi[s]) along `axis` instead of the launch's box.
+// A listed launch (the listed z-slab form) runs over the concatenation of the
+// k_zclass lists list[0 .. nseg) (list l: lists + l * cap, length counts[l]; indices into
+// `events` and `fp`), in order. box = 1: an event of segment s is clipped to [lo[s], hi[s])
+// along `axis` instead of the launch's box (windows, or a coarse slab among windows).
 constexpr int kMaxSeg = 8;
 struct ListArg {
     const int* lists;
     const int* counts;
     long long cap;
-    int first, nseg, axis, box;
-    int lo[kMaxSeg], hi[kMaxSeg];
+    int nseg, axis, box;
+    int list[kMaxSeg], lo[kMaxSeg], hi[kMaxSeg];
 };
 
 // LIST (MODEs 2, 3, 5, 6): the launch runs over the listed events of `la` instead of [0, n).
@@ -547,16 +547,18 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     // fewer than 4, >= 4; guided divisor 3 from 6 rounds of 32-event claims, else 2)
     // ends of the segments in the concatenation, and their clip planes (static indices here:
     // a dynamic index into the parameter array would copy it to the stack)
-    __shared__ int s_segend[LIST ? kMaxSeg : 1], s_seglo[LIST ? kMaxSeg : 1], s_seghi[LIST ? kMaxSeg : 1];
+    __shared__ int s_segend[LIST ? kMaxSeg : 1], s_seglo[LIST ? kMaxSeg : 1], s_seghi[LIST ? kMaxSeg : 1],
+        s_seglist[LIST ? kMaxSeg : 1];
     if (LIST) {
         int acc = 0;
 #pragma unroll
         for (int q = 0; q < kMaxSeg; ++q) {
-            if (q < la.nseg) acc += __ldg(la.counts + la.first + q);
+            if (q < la.nseg) acc += __ldg(la.counts + la.list[q]);
             if (threadIdx.x == 0) {
                 s_segend[q] = acc;
                 s_seglo[q] = la.lo[q];
                 s_seghi[q] = la.hi[q];
+                s_seglist[q] = la.list[q];
             }
         }
         __syncthreads();
@@ -604,7 +606,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             if (mine_ev) {
                 int lo_i = 0;
                 while (sg < la.nseg - 1 && idx >= s_segend[sg]) lo_i = s_segend[sg++];
-                eidx = (int64_t)__ldg(la.lists + (int64_t)(la.first + sg) * la.cap + (idx - lo_i));
+                eidx = (int64_t)__ldg(la.lists + (int64_t)s_seglist[sg] * la.cap + (idx - lo_i));
             }
         }
         // event tile staging: the claimed events (24 B each, contiguous) are loaded with
@@ -781,11 +783,27 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
 // list. Lists: lists + l * cap, lengths counts[l]; l < K coarse, K <= l < K + Kf fine.
 constexpr int kZMaxLists = 32;
 struct ZClass {
-    int K, Kf, axis;
+    int K, Kf, Km, axis;
     int cb[kZMaxLists + 1];  // coarse slab planes (voxels along axis): cb[0] = 0 .. cb[K] = n
     int wlo[kZMaxLists], whi[kZMaxLists];  // fine windows [wlo, whi): wlo = j * ws (the last
     float ws, ww, wlast;                   // one: wlast), whi = wlo + ww
+    float ms, mw, mlast;                   // medium windows (coarse-slab wide), the same way
 };
+
+// The window of a family (starts j * stride, the last one at `last`; width w; cnt windows)
+// that holds [zl, zh] kZMarginF clear of its planes, or -1. The window starting last at or
+// below zl - m is the only candidate (earlier ones end earlier), besides the clamped last one.
+__device__ __forceinline__ int win_fit(float zl, float zh, float m, float stride, float w, float last, int cnt) {
+    if (cnt <= 0) return -1;
+    const int j = min((int)floorf(fmaxf(zl - m, 0.0f) / stride), cnt - 1);
+    const float lo = j == cnt - 1 ? last : (float)j * stride;
+    if (zl >= lo + m && zh <= lo + w - m) return j;
+    if (j > 0 && j == cnt - 1) {  // the last window may start below the stride grid
+        const float lo2 = (float)(j - 1) * stride;
+        if (zl >= lo2 + m && zh <= lo2 + w - m) return j - 1;
+    }
+    return -1;
+}
 
 // Membership bits of one event (bit l set: the event goes to list l), in float32 against a
 // box grown by kZMarginF voxels, so the clipped range contains the float64 one (lor_setup)
@@ -833,17 +851,10 @@ __device__ __forceinline__ unsigned zclass_bits(const float ev[6], const GridGeo
     const float za = fmaf(amin, Ds, us), zb = fmaf(amax, Ds, us);
     const float zl = fminf(za, zb), zh = fmaxf(za, zb);
     if (!isfinite(zl) || !isfinite(zh)) return all;
-    if (zc.Kf > 0) {
-        // the window starting last at or below zl - m is the only candidate (earlier ones
-        // end earlier), and the clamped last window
-        const int j = min((int)floorf(fmaxf(zl - m, 0.0f) / zc.ws), zc.Kf - 1);
-        const float lo = j == zc.Kf - 1 ? zc.wlast : (float)j * zc.ws;
-        if (zl >= lo + m && zh <= lo + zc.ww - m) return 1u << (zc.K + j);
-        if (j > 0 && j == zc.Kf - 1) {  // the last window may start below the stride grid
-            const float lo2 = (float)(j - 1) * zc.ws;
-            if (zl >= lo2 + m && zh <= lo2 + zc.ww - m) return 1u << (zc.K + j - 1);
-        }
-    }
+    const int jf = win_fit(zl, zh, m, zc.ws, zc.ww, zc.wlast, zc.Kf);
+    if (jf >= 0) return 1u << (zc.K + jf);
+    const int jm = win_fit(zl, zh, m, zc.ms, zc.mw, zc.mlast, zc.Km);
+    if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);
     unsigned bits = 0u;
     for (int k = 0; k < zc.K; ++k)
         if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) bits |= 1u << k;
@@ -866,7 +877,7 @@ __global__ void __launch_bounds__(kZThreads) k_zclass(const float* __restrict__ 
     pdl_wait();
     pdl_trigger();
     __shared__ int s_cnt[kZMaxLists], s_base[kZMaxLists];
-    const int nl = zc.K + zc.Kf;
+    const int nl = zc.K + zc.Kf + zc.Km;
     for (int64_t c0 = (int64_t)blockIdx.x * kZChunk; c0 < n; c0 += (int64_t)gridDim.x * kZChunk) {
         if ((int)threadIdx.x < nl) s_cnt[threadIdx.x] = 0;
         __syncthreads();

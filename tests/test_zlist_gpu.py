@@ -56,22 +56,23 @@ def subset_case(name):
 
 
 # (LMOSEM_ZLIST, ZFINE windows per coarse slab, ZFUSED_MODE, ZOVER window overlap, ZWIN width,
-#  ZMERGE: the windows of a coarse slab in one launch)
-FORMS = [("0", "2", "6", "1", "0", "1"), ("1", "2", "6", "1", "0", "1"), ("2", "2", "6", "1", "0", "1"),
-         ("2", "1", "6", "1", "0", "1"), ("2", "3", "5", "1", "0", "1"), ("2", "2", "6", "2", "0", "1"),
-         ("2", "3", "6", "3", "0", "1"), ("2", "2", "5", "2", "0", "0"), ("2", "2", "5", "2", "20", "1"),
-         ("2", "2", "5", "4", "8", "1")]
+#  ZMERGE: the windows of a coarse slab in one launch, ZMED: medium-window stride divisor, 0 = none)
+FORMS = [("0", "2", "6", "1", "0", "1", "3"), ("1", "2", "6", "1", "0", "1", "0"), ("1", "2", "6", "1", "0", "1", "3"),
+         ("2", "2", "6", "1", "0", "1", "0"), ("2", "1", "6", "1", "0", "1", "3"), ("2", "3", "5", "1", "0", "1", "2"),
+         ("2", "2", "6", "2", "0", "1", "3"), ("2", "3", "6", "3", "0", "1", "1"), ("2", "2", "5", "2", "0", "0", "3"),
+         ("2", "2", "5", "2", "20", "1", "3"), ("2", "2", "5", "4", "8", "1", "3"), ("2", "2", "5", "4", "0", "1", "8")]
 
 
-@pytest.mark.parametrize("zlist,zfine,zmode,zover,zwin,zmerge", FORMS)
+@pytest.mark.parametrize("zlist,zfine,zmode,zover,zwin,zmerge,zmed", FORMS)
 @pytest.mark.parametrize("name,slabs", [("C1", 2), ("C1", 3), ("C1", 5), ("C2", 3)])
-def test_listed_zslab_subset_matches_oracle(pkg, monkeypatch, zlist, zfine, zmode, zover, zwin, zmerge, name,
+def test_listed_zslab_subset_matches_oracle(pkg, monkeypatch, zlist, zfine, zmode, zover, zwin, zmerge, zmed, name,
                                             slabs):
     """ZWIN=20 at C2 with 3 slabs: 27 windows, 9 centred in a coarse slab -> two merged launches
     (kMaxSeg = 8); ZWIN=8 at stride 2 would need > 32 lists at C2: the stride grows until they
-    fit; C1 with 5 slabs runs the unlisted form (listed needs <= 4 coarse slabs)."""
+    fit; ZMED=8 leaves no list budget for medium windows at C2 (none are made); C1 with 5
+    slabs runs the unlisted form (listed needs <= 4 coarse slabs)."""
     for k, v in (("ZLIST", zlist), ("ZFINE", zfine), ("ZFUSED_MODE", zmode), ("ZOVER", zover), ("ZWIN", zwin),
-                 ("ZMERGE", zmerge)):
+                 ("ZMERGE", zmerge), ("ZMED", zmed)):
         monkeypatch.setenv("LMOSEM_" + k, v)
     cfg, ev, s, f0, ref = subset_case(name)
     rec = pkg.Reconstructor(cfg.dims, cfg.voxel_mm, dev(s))
@@ -112,12 +113,14 @@ def plane_events(dims, vox):
     return np.array(out, np.float32)
 
 
-@pytest.mark.parametrize("zlist,zover,zmerge", [("0", "1", "1"), ("1", "1", "1"), ("2", "1", "1"), ("2", "2", "1"),
-                                               ("2", "2", "0")])
-def test_listed_zslab_plane_cases(pkg, monkeypatch, zlist, zover, zmerge):
+@pytest.mark.parametrize("zlist,zover,zmerge,zmed", [("0", "1", "1", "3"), ("1", "1", "1", "0"), ("1", "1", "1", "3"),
+                                                    ("2", "1", "1", "0"), ("2", "2", "1", "3"), ("2", "2", "0", "1"),
+                                                    ("2", "4", "1", "3")])
+def test_listed_zslab_plane_cases(pkg, monkeypatch, zlist, zover, zmerge, zmed):
     monkeypatch.setenv("LMOSEM_ZLIST", zlist)
     monkeypatch.setenv("LMOSEM_ZOVER", zover)
     monkeypatch.setenv("LMOSEM_ZMERGE", zmerge)
+    monkeypatch.setenv("LMOSEM_ZMED", zmed)
     cfg = lmgen.CONFIGS["C1"]
     ev = plane_events(cfg.dims, cfg.voxel_mm)
     g = oracle.geom(cfg.dims, cfg.voxel_mm)

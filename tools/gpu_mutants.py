@@ -85,13 +85,15 @@ MUTANTS = [
     ("fused combine: local c not re-zeroed", K, "            C[2 * b] = z;\n            C[2 * b + 1] = z;\n", "", False),
     ("fused combine: second brick of a pair not stored", K, "            team.store_f(ob, nb0, nb1);\n", "", False),
     # the listed z-slab form (round 2: caught by tests/test_zlist_gpu.py and the loopback test)
-    ("listed: window membership without its margin", K, "if (zl >= lo + m && zh <= lo + zc.ww - m) return",
-     "if (zl >= lo - m && zh <= lo + zc.ww + m) return", False),
+    ("listed: window membership without its margin", K, "if (zl >= lo + m && zh <= lo + w - m) return j;",
+     "if (zl >= lo - m && zh <= lo + w + m) return j;", False),
     ("listed: coarse membership shrunk by the margin", K,
      "if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) bits |= 1u << k;",
      "if (zh > (float)zc.cb[k] + m && zl < (float)zc.cb[k + 1] - m) bits |= 1u << k;", False),
-    ("listed: window LORs also in the coarse lists", K, "return 1u << (zc.K + j);", "return (1u << (zc.K + j)) | all;",
-     False),
+    ("listed: window LORs also in the coarse lists", K, "if (jf >= 0) return 1u << (zc.K + jf);",
+     "if (jf >= 0) return (1u << (zc.K + jf)) | all;", False),
+    ("listed: medium-window LORs also in the coarse lists", K, "if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);",
+     "if (jm >= 0) return (1u << (zc.K + zc.Kf + jm)) | all;", False),
     ("listed: list slots without the per-event offset", K, "lists[(int64_t)l * cap + s_base[l] + off[p][q]] = e;",
      "lists[(int64_t)l * cap + s_base[l]] = e;", False),
     ("listed: segment lookup off by one", K, "while (sg < la.nseg - 1 && idx >= s_segend[sg])",

@@ -11,9 +11,9 @@ for rep in 1 2; do
  IFS=',' read -ra FORMS <<< "${ZAB_FORMS:-0_2_6_1,1_2_6_1,2_2_6_1,2_2_6_2,2_3_6_2,2_2_5_2}"
  for v in "${FORMS[@]}"; do
   set -- ${v//_/ }
-  T=$1_$2_$3_$4_${5:-0}_${6:-1}_r$rep
-  LMOSEM_ZLIST=$1 LMOSEM_ZFINE=$2 LMOSEM_ZFUSED_MODE=$3 LMOSEM_ZOVER=$4 LMOSEM_ZWIN=${5:-0} LMOSEM_ZMERGE=${6:-1} timeout 300 python bench.py --config C4 --steps 10 --no-cpu-baseline --no-e2e > $O/b_$T.json 2>$O/b_$T.err
-  python -c "import json;d=json.load(open('$O/b_$T.json'));print('C4 zlist=$1 zfine=$2 mode=$3 zover=$4 zwin=${5:-0} zmerge=${6:-1}', round(d['ms_per_step'],3), d['phase_ms_per_step'].get('project'))" 2>&1 | tail -1
+  T=$1_$2_$3_$4_${5:-0}_${6:-1}_${7:-3}_r$rep
+  LMOSEM_ZLIST=$1 LMOSEM_ZFINE=$2 LMOSEM_ZFUSED_MODE=$3 LMOSEM_ZOVER=$4 LMOSEM_ZWIN=${5:-0} LMOSEM_ZMERGE=${6:-1} LMOSEM_ZMED=${7:-3} timeout 300 python bench.py --config C4 --steps 10 --no-cpu-baseline --no-e2e > $O/b_$T.json 2>$O/b_$T.err
+  python -c "import json;d=json.load(open('$O/b_$T.json'));print('C4 zlist=$1 zfine=$2 mode=$3 zover=$4 zwin=${5:-0} zmerge=${6:-1} zmed=${7:-3}', round(d['ms_per_step'],3), d['phase_ms_per_step'].get('project'))" 2>&1 | tail -1
  done
 done
 M=gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum,lts__t_sector_hit_rate.pct,sm__inst_executed.sum
