@@ -440,6 +440,9 @@ constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 constexpr unsigned kLorRecBytes = 80;
 __host__ __device__ constexpr bool lor_in_smem(int mode) { return mode == 2 || mode == 3; }
 __host__ __device__ constexpr size_t lor_bytes_per_warp(int mode) { return 32u * (lor_in_smem(mode) ? kLorRecBytes : 24u); }
+#ifndef LMK_LATE_WAIT
+#define LMK_LATE_WAIT 1  // listed pass A / window launches wait for their predecessor at exit (A/B)
+#endif
 #ifndef LMK_GEOM_UNROLL
 #define LMK_GEOM_UNROLL 0  // unroll of the geometry loop (0 = the compiler's choice, 2x)
 #endif
@@ -571,7 +574,14 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
     pdl_trigger();
     // claims, event tiles and the float64 setup of the first LORs overlap the previous
     // kernel's tail; pass B reads fp during setup, so it waits at once
-    bool dep_ready = MODE == 3;
+    // A listed pass A or window launch (kLateWait) depends on no earlier listed launch of the
+    // subset: it reads f (final before the plain launch that starts the sequence) and adds into
+    // c and fp with atomics. So it waits for its predecessor only before exiting, and overlaps
+    // the predecessor's tail with real work. Its completion still implies the predecessor's,
+    // so pass B (which waits at entry for the fp of every pass A) and the kernel after the
+    // sequence see all of it complete.
+    constexpr bool kLateWait = LIST && LMK_LATE_WAIT && MODE != 3;
+    bool dep_ready = MODE == 3 || kLateWait;
     if (MODE == 3) pdl_wait();
 #if LMK_TRACE
     const int gw = blockIdx.x * (blockDim.x >> 5) + wib;
@@ -748,7 +758,12 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 fpv = warp_sum(acc) * L.lunit;
                 const int64_t esrc = LIST ? (int64_t)__shfl_sync(0xffffffffu, (int)eidx, src) : base + src;
                 if (MODE == 1 && lane == 0) fp[esrc] = fpv;
-                if (MODE == 2 && lane == 0) fp[esrc] += fpv;
+                if (MODE == 2 && lane == 0) {
+                    if (kLateWait)
+                        atomicAdd(fp + esrc, fpv);  // pass A launches of a LOR's slabs may overlap
+                    else
+                        fp[esrc] += fpv;
+                }
             } else {
                 fpv = __shfl_sync(0xffffffffu, fp_known, src);
             }
@@ -766,6 +781,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             __syncwarp();
         }
     }
+    if (kLateWait) pdl_wait();
 }
 
 // ------------------------------------------------------------ listed z-slab form (C4)
