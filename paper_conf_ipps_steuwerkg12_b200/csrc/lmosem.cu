@@ -743,6 +743,7 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
             la.cap = ctx->zlist_cap;
             la.axis = zc.axis;
             la.box = 1;
+            la.entry_wait = mode == 3 && k == 0 && i == 0;  // the first pass B waits for every pass A
             la.nseg = (int)std::min<size_t>(lmk::kMaxSeg, segs.size() - i);
             int widest = 0;
             for (int q = 0; q < la.nseg; ++q) {

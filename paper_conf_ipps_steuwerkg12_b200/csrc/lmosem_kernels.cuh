@@ -511,6 +511,7 @@ struct ListArg {
     const int* counts;
     long long cap;
     int nseg, axis, box;
+    int entry_wait;  // pass B: wait for the predecessor at entry (the first pass B of a subset)
     int list[kMaxSeg], lo[kMaxSeg], hi[kMaxSeg];
 };
 
@@ -571,18 +572,20 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
         batch = take;
         gdiv = n >= 6 * 32 * warps_in_grid ? 3 : 2;
     }
-    pdl_trigger();
     // claims, event tiles and the float64 setup of the first LORs overlap the previous
-    // kernel's tail; pass B reads fp during setup, so it waits at once
-    // A listed pass A or window launch (kLateWait) depends on no earlier listed launch of the
+    // kernel's tail; pass B reads fp during setup, so it waits at once — the first listed
+    // pass B of a subset before it lets its dependents launch, so that every later listed
+    // launch starts after all of pass A has completed and may wait late (late_wait)
+    // A listed pass A or window launch (late_wait) depends on no earlier listed launch of the
     // subset: it reads f (final before the plain launch that starts the sequence) and adds into
-    // c and fp with atomics. So it waits for its predecessor only before exiting, and overlaps
-    // the predecessor's tail with real work. Its completion still implies the predecessor's,
-    // so pass B (which waits at entry for the fp of every pass A) and the kernel after the
-    // sequence see all of it complete.
-    constexpr bool kLateWait = LIST && LMK_LATE_WAIT && MODE != 3;
-    bool dep_ready = MODE == 3 || kLateWait;
-    if (MODE == 3) pdl_wait();
+    // c and fp with atomics; a listed pass B after the first one starts only once every pass A
+    // has completed (above). So they wait for their predecessor only before exiting, and
+    // overlap its tail with real work. A launch's completion still implies its predecessor's,
+    // so the first pass B and the kernel after the sequence see all of it complete.
+    const bool late_wait = LIST && LMK_LATE_WAIT && !(MODE == 3 && la.entry_wait);
+    bool dep_ready = MODE == 3 || late_wait;
+    if (MODE == 3 && !late_wait) pdl_wait();
+    pdl_trigger();
 #if LMK_TRACE
     const int gw = blockIdx.x * (blockDim.x >> 5) + wib;
     unsigned long long tr_start = gtimer(), tr_first = 0, tr_lors = 0, tr_claims = 0;
@@ -759,7 +762,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                 const int64_t esrc = LIST ? (int64_t)__shfl_sync(0xffffffffu, (int)eidx, src) : base + src;
                 if (MODE == 1 && lane == 0) fp[esrc] = fpv;
                 if (MODE == 2 && lane == 0) {
-                    if (kLateWait)
+                    if (late_wait)
                         atomicAdd(fp + esrc, fpv);  // pass A launches of a LOR's slabs may overlap
                     else
                         fp[esrc] += fpv;
@@ -781,7 +784,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
             __syncwarp();
         }
     }
-    if (kLateWait) pdl_wait();
+    if (late_wait) pdl_wait();
 }
 
 // ------------------------------------------------------------ listed z-slab form (C4)
