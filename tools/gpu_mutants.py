@@ -92,8 +92,10 @@ MUTANTS = [
      "if (zh > (float)zc.cb[k] + m && zl < (float)zc.cb[k + 1] - m) bits |= 1u << k;", False),
     ("listed: window LORs also in the coarse lists", K, "if (jf >= 0) return 1u << (zc.K + jf);",
      "if (jf >= 0) return (1u << (zc.K + jf)) | all;", False),
-    ("listed: medium-window LORs also in the coarse lists", K, "if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);",
-     "if (jm >= 0) return (1u << (zc.K + zc.Kf + jm)) | all;", False),
+    ("listed: medium-window LORs in no list", K, "if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);",
+     "if (jm >= 0) return 0u;", False),
+    ("listed: medium window of the next family index", K, "if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);",
+     "if (jm >= 0) return 1u << (zc.K + zc.Kf + min(jm + 1, zc.Km - 1));", False),
     ("listed: list slots without the per-event offset", K, "lists[(int64_t)l * cap + s_base[l] + off[p][q]] = e;",
      "lists[(int64_t)l * cap + s_base[l]] = e;", False),
     ("listed: segment lookup off by one", K, "while (sg < la.nseg - 1 && idx >= s_segend[sg])",
@@ -101,7 +103,9 @@ MUTANTS = [
     ("listed: window box not applied per event", K, "const bool w = LIST && la.box && k == la.axis;",
      "const bool w = false;", False),
 ]
-# Not listed: equivalent mutants. Dropping the 2^-40 offset of the mirrored frame changes
+# Not listed: equivalent mutants. A medium-window LOR also put in every coarse list is
+# projected twice in pass A (its whole path in the window, its pieces per slab: fp doubles) and
+# back-projected twice with that fp, so c is unchanged (measured: it survives, as expected). Dropping the 2^-40 offset of the mirrored frame changes
 # only exactly integral up-moving positions, where "voxel m - 1 with a crossing at d = 0"
 # yields the same pieces as "voxel m, no crossing" (the zero-length piece is dropped); and
 # any change to the ISD rank block (b0 = chunk * rank) is invisible at world size 1, the only
