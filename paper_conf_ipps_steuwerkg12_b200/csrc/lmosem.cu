@@ -111,7 +111,7 @@ struct lmosem_ctx {
     int zover = 4;             // fine windows overlap: stride = width / zover (LMOSEM_ZOVER)
     int zwin = 0;              // fine window width in voxels (LMOSEM_ZWIN; 0: from zfine_per)
     int zmerge = 1;            // the windows of a coarse slab in one launch (LMOSEM_ZMERGE)
-    int zmed = 3;              // medium windows: stride = coarse width / zmed (LMOSEM_ZMED; 0: none)
+    int zmed = 6;              // medium windows: stride = coarse width / zmed (LMOSEM_ZMED; 0: none)
     int* zlist = nullptr;      // lists, zlist_cap indices each
     int* zcount = nullptr;     // their lengths (kZMaxLists)
     int64_t zlist_cap = 0;
@@ -1422,7 +1422,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (const char* e = std::getenv("LMOSEM_ZOVER")) ctx->zover = std::max(1, std::min(4, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_ZWIN")) ctx->zwin = std::max(0, std::atoi(e));
     if (const char* e = std::getenv("LMOSEM_ZMERGE")) ctx->zmerge = e[0] != '0';
-    if (const char* e = std::getenv("LMOSEM_ZMED")) ctx->zmed = std::max(0, std::min(8, std::atoi(e)));
+    if (const char* e = std::getenv("LMOSEM_ZMED")) ctx->zmed = std::max(0, std::min(16, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {

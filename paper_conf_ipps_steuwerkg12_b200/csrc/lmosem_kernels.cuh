@@ -505,7 +505,7 @@ __host__ __device__ constexpr int proj_threads_of(int mode) {
 // k_zclass lists list[0 .. nseg) (list l: lists + l * cap, length counts[l]; indices into
 // `events` and `fp`), in order. box = 1: an event of segment s is clipped to [lo[s], hi[s])
 // along `axis` instead of the launch's box (windows, or a coarse slab among windows).
-constexpr int kMaxSeg = 8;
+constexpr int kMaxSeg = 16;
 struct ListArg {
     const int* lists;
     const int* counts;
@@ -800,7 +800,7 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
 //     and B over slab k; a listed LOR that misses the slab is dropped by its clip).
 // An event that cannot contribute (non-finite, zero length, missing the volume) is in no
 // list. Lists: lists + l * cap, lengths counts[l]; l < K coarse, K <= l < K + Kf fine.
-constexpr int kZMaxLists = 32;
+constexpr int kZMaxLists = 64;
 struct ZClass {
     int K, Kf, Km, axis;
     int cb[kZMaxLists + 1];  // coarse slab planes (voxels along axis): cb[0] = 0 .. cb[K] = n
@@ -824,7 +824,8 @@ __device__ __forceinline__ int win_fit(float zl, float zh, float m, float stride
     return -1;
 }
 
-// Membership bits of one event (bit l set: the event goes to list l), in float32 against a
+// The lists of one event, as a code (first list << 4) | count (0: none): one window list, or
+// the contiguous run of coarse slabs its range meets. Decided in float32 against a
 // box grown by kZMarginF voxels, so the clipped range contains the float64 one (lor_setup)
 // up to float32 rounding (< 1e-2 voxel while both ends lie within 2 volume extents of the
 // centre; farther or non-finite LORs go to every coarse list, where lor_setup decides):
@@ -832,9 +833,10 @@ __device__ __forceinline__ int win_fit(float zl, float zh, float m, float stride
 //   - a coarse list gets every LOR whose grown range meets the slab (a superset);
 //   - no list: clearly zero length or missing the grown box.
 constexpr float kZMarginF = 0.02f;
+__device__ __forceinline__ unsigned zlist_code(int first, int count) { return ((unsigned)first << 4) | (unsigned)count; }
 __device__ __forceinline__ unsigned zclass_bits(const float ev[6], const GridGeom& g, const ZClass& zc) {
     constexpr float m = kZMarginF;
-    const unsigned all = (1u << zc.K) - 1u;
+    const unsigned all = zlist_code(0, zc.K);
     const float nmax = (float)max(g.n[0], max(g.n[1], g.n[2]));
     float u1[3], D[3];
     bool far = false, zero = true;
@@ -871,13 +873,16 @@ __device__ __forceinline__ unsigned zclass_bits(const float ev[6], const GridGeo
     const float zl = fminf(za, zb), zh = fmaxf(za, zb);
     if (!isfinite(zl) || !isfinite(zh)) return all;
     const int jf = win_fit(zl, zh, m, zc.ws, zc.ww, zc.wlast, zc.Kf);
-    if (jf >= 0) return 1u << (zc.K + jf);
+    if (jf >= 0) return zlist_code(zc.K + jf, 1);
     const int jm = win_fit(zl, zh, m, zc.ms, zc.mw, zc.mlast, zc.Km);
-    if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);
-    unsigned bits = 0u;
+    if (jm >= 0) return zlist_code(zc.K + zc.Kf + jm, 1);
+    int k0 = zc.K, k1 = -1;  // the coarse slabs met form one run
     for (int k = 0; k < zc.K; ++k)
-        if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) bits |= 1u << k;
-    return bits;
+        if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) {
+            k0 = min(k0, k);
+            k1 = k;
+        }
+    return k1 >= k0 ? zlist_code(k0, k1 - k0 + 1) : 0u;
 }
 
 // One CTA per chunk of kZChunk consecutive events (grid-stride): each event takes its slot in
@@ -914,28 +919,21 @@ __global__ void __launch_bounds__(kZThreads) k_zclass(const float* __restrict__ 
         int off[kZPer][kZMaxBits];
 #pragma unroll
         for (int p = 0; p < kZPer; ++p) {
-            unsigned b = bits[p];
+            const int l0 = (int)(bits[p] >> 4), cnt = (int)(bits[p] & 15u);
 #pragma unroll
-            for (int q = 0; q < kZMaxBits; ++q) {
-                if (b) off[p][q] = atomicAdd(&s_cnt[__ffs(b) - 1], 1);
-                b &= b - 1;
-            }
+            for (int q = 0; q < kZMaxBits; ++q)
+                if (q < cnt) off[p][q] = atomicAdd(&s_cnt[l0 + q], 1);
         }
         __syncthreads();
         if ((int)threadIdx.x < nl) s_base[threadIdx.x] = s_cnt[threadIdx.x] ? atomicAdd(counts + threadIdx.x, s_cnt[threadIdx.x]) : 0;
         __syncthreads();
 #pragma unroll
         for (int p = 0; p < kZPer; ++p) {
-            unsigned b = bits[p];
+            const int l0 = (int)(bits[p] >> 4), cnt = (int)(bits[p] & 15u);
             const int e = (int)(c0 + p * kZThreads + threadIdx.x);
 #pragma unroll
-            for (int q = 0; q < kZMaxBits; ++q) {
-                if (b) {
-                    const int l = __ffs(b) - 1;
-                    lists[(int64_t)l * cap + s_base[l] + off[p][q]] = e;
-                }
-                b &= b - 1;
-            }
+            for (int q = 0; q < kZMaxBits; ++q)
+                if (q < cnt) lists[(int64_t)(l0 + q) * cap + s_base[l0 + q] + off[p][q]] = e;
         }
         __syncthreads();  // s_cnt / s_base are rewritten by the next chunk
     }

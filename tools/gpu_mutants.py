@@ -88,16 +88,17 @@ MUTANTS = [
     ("listed: window membership without its margin", K, "if (zl >= lo + m && zh <= lo + w - m) return j;",
      "if (zl >= lo - m && zh <= lo + w + m) return j;", False),
     ("listed: coarse membership shrunk by the margin", K,
-     "if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) bits |= 1u << k;",
-     "if (zh > (float)zc.cb[k] + m && zl < (float)zc.cb[k + 1] - m) bits |= 1u << k;", False),
-    ("listed: window LORs also in the coarse lists", K, "if (jf >= 0) return 1u << (zc.K + jf);",
-     "if (jf >= 0) return (1u << (zc.K + jf)) | all;", False),
-    ("listed: medium-window LORs in no list", K, "if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);",
+     "if (zh + m > (float)zc.cb[k] && zl - m < (float)zc.cb[k + 1]) {",
+     "if (zh > (float)zc.cb[k] + m && zl < (float)zc.cb[k + 1] - m) {", False),
+    ("listed: window LORs also in the coarse lists", K, "if (jf >= 0) return zlist_code(zc.K + jf, 1);",
+     "if (jf >= 0) return zlist_code(0, zc.K + jf + 1);", False),
+    ("listed: medium-window LORs in no list", K, "if (jm >= 0) return zlist_code(zc.K + zc.Kf + jm, 1);",
      "if (jm >= 0) return 0u;", False),
-    ("listed: medium window of the next family index", K, "if (jm >= 0) return 1u << (zc.K + zc.Kf + jm);",
-     "if (jm >= 0) return 1u << (zc.K + zc.Kf + min(jm + 1, zc.Km - 1));", False),
-    ("listed: list slots without the per-event offset", K, "lists[(int64_t)l * cap + s_base[l] + off[p][q]] = e;",
-     "lists[(int64_t)l * cap + s_base[l]] = e;", False),
+    ("listed: medium window of the next family index", K, "if (jm >= 0) return zlist_code(zc.K + zc.Kf + jm, 1);",
+     "if (jm >= 0) return zlist_code(zc.K + zc.Kf + min(jm + 1, zc.Km - 1), 1);", False),
+    ("listed: list slots without the per-event offset", K,
+     "if (q < cnt) lists[(int64_t)(l0 + q) * cap + s_base[l0 + q] + off[p][q]] = e;",
+     "if (q < cnt) lists[(int64_t)(l0 + q) * cap + s_base[l0 + q]] = e;", False),
     ("listed: segment lookup off by one", K, "while (sg < la.nseg - 1 && idx >= s_segend[sg])",
      "while (sg < la.nseg - 1 && idx > s_segend[sg])", False),
     ("listed: window box not applied per event", K, "const bool w = LIST && la.box && k == la.axis;",
