@@ -198,11 +198,12 @@ int32_t lmosem_get_combine(const lmosem_ctx* ctx);
  * slabs are then never longer than 1170 (at least that many slabs whatever is asked).
  * With 2-4 slabs and fewer than 2^31 events per call the passes are listed (the default,
  * LMOSEM_ZLIST=2): one classification kernel per subset sorts the events into per-launch
- * index lists, LORs inside one of the overlapping fine windows (about a quarter of a slab
- * wide, fine enough that the window's f and c fit L2 together) are projected by one fused
- * pass over their window, and the others by passes A and B over only the slabs they cross.
- * The lists take 4 B x events x (slabs + windows) of device memory, allocated on first use
- * and kept with the context (C4, 10^7 events: 0.96 GB); ENOMEM if that fails.
+ * index lists. LORs inside one of the overlapping fine windows (about half a slab wide, fine
+ * enough that the window's f and c fit L2 together) are projected by one fused pass over
+ * their window; LORs inside one of the overlapping slab-wide windows by passes A and B over
+ * that window; the others by passes A and B over only the slabs they cross. The lists take
+ * 4 B x events x (slabs + windows) of device memory, allocated on first use and kept with
+ * the context (C4, 10^7 events, 3 + 22 + 13 lists: 1.5 GB); ENOMEM if that fails.
  * The result is the same up to fp32 rounding. EINVAL if n_slabs < 0. */
 lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs);
 
