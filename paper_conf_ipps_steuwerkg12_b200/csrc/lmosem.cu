@@ -671,12 +671,16 @@ lmk::GridGeom slab_geom(const lmosem_ctx* ctx, int k, int K) {
     return g;
 }
 
-// The listed z-slab form of step 1: k_zclass sorts the n events into the
-// coarse lists X_k (LORs that leave a fine slab: passes A and B over coarse slab k only for
-// the LORs that meet it) and the fine lists F_j (LORs inside fine slab j: one fused launch
-// over the fine slab box, whose f and c slabs fit L2 together). Order: pass A over every
-// coarse slab (fp of the X LORs complete), then per coarse slab k the fused launches of its
-// fine slabs and pass B of X_k, so c's slab k stays L2-resident across them.
+// The listed z-slab form of step 1: k_zclass sorts the n events into
+//   - the fine-window lists F_j (`wins`; LORs inside fine window j: one fused pass over the
+//     window box, whose f and c fit L2 together),
+//   - the medium-window lists M_j (`mwins`, coarse-slab wide; LORs inside one: passes A and B
+//     over that window only),
+//   - the coarse lists X_k (the other LORs: passes A and B over each coarse slab they meet).
+// Order: pass A of every coarse slab k over [X_k, the M_j centred in slab k] (fp complete),
+// then per coarse slab k one fused launch over the F_j centred in it and pass B over
+// [X_k, M_j centred in it], so c's slab k stays L2-resident across them. The listed launches
+// wait for their predecessor at exit (k_project, late_wait), except the first pass B.
 lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n, int K,
                                    const std::vector<std::pair<int, int>>& wins,
                                    const std::vector<std::pair<int, int>>& mwins) {
