@@ -112,6 +112,7 @@ struct lmosem_ctx {
     int zwin = 0;              // fine window width in voxels (LMOSEM_ZWIN; 0: from zfine_per)
     int zmerge = 1;            // the windows of a coarse slab in one launch (LMOSEM_ZMERGE)
     int zmed = 6;              // medium windows: stride = coarse width / zmed (LMOSEM_ZMED; 0: none)
+    int zamerge = 0;           // pass A of all coarse slabs in shared launches (LMOSEM_ZAMERGE)
     int* zlist = nullptr;      // lists, zlist_cap indices each
     int* zcount = nullptr;     // their lengths (kZMaxLists)
     int64_t zlist_cap = 0;
@@ -735,11 +736,15 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
     };
     // passes A / B of region k: coarse slab k's list, then the medium windows centred in it
     // (each event clipped to its own segment's box; the path buffers sized for the widest)
-    auto two_pass = [&](int mode, int k) -> lmosem_status {
+    // k0..k1: the regions in one launch sequence (pass A of all regions may share launches)
+    auto two_pass = [&](int mode, int k0, int k1) -> lmosem_status {
         struct Seg { int list, lo, hi; };
-        std::vector<Seg> segs{{k, zc.cb[k], zc.cb[k + 1]}};
-        for (int j = 0; j < Km; ++j)
-            if (in_slab(mwins[j], k)) segs.push_back({K + Kf + j, mwins[j].first, mwins[j].second});
+        std::vector<Seg> segs;
+        for (int k = k0; k <= k1; ++k) {
+            segs.push_back({k, zc.cb[k], zc.cb[k + 1]});
+            for (int j = 0; j < Km; ++j)
+                if (in_slab(mwins[j], k)) segs.push_back({K + Kf + j, mwins[j].first, mwins[j].second});
+        }
         for (size_t i = 0; i < segs.size(); i += lmk::kMaxSeg) {
             lmk::ListArg la{};
             la.lists = ctx->zlist;
@@ -747,7 +752,7 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
             la.cap = ctx->zlist_cap;
             la.axis = zc.axis;
             la.box = 1;
-            la.entry_wait = mode == 3 && k == 0 && i == 0;  // the first pass B waits for every pass A
+            la.entry_wait = mode == 3 && k0 == 0 && i == 0;  // the first pass B waits for every pass A
             la.nseg = (int)std::min<size_t>(lmk::kMaxSeg, segs.size() - i);
             int widest = 0;
             for (int q = 0; q < la.nseg; ++q) {
@@ -763,8 +768,12 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
         }
         return LMOSEM_OK;
     };
-    for (int k = 0; k < K; ++k)
-        if ((s = two_pass(2, k))) return s;
+    if (ctx->zamerge) {  // pass A of every region in as few launches as kMaxSeg allows
+        if ((s = two_pass(2, 0, K - 1))) return s;
+    } else {
+        for (int k = 0; k < K; ++k)
+            if ((s = two_pass(2, k, k))) return s;
+    }
     const int fused = ctx->zfused_mode;
     for (int k = 0; k < K; ++k) {
         // the windows centred in slab k, in order, as one launch (up to kMaxSeg per launch, or
@@ -794,7 +803,7 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
             }
             if ((s = launch_mode(ctx, fused, evf, n, nullptr, gj, &la))) return s;
         }
-        if ((s = two_pass(3, k))) return s;
+        if ((s = two_pass(3, k, k))) return s;
     }
     return LMOSEM_OK;
 }
@@ -1427,6 +1436,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (const char* e = std::getenv("LMOSEM_ZWIN")) ctx->zwin = std::max(0, std::atoi(e));
     if (const char* e = std::getenv("LMOSEM_ZMERGE")) ctx->zmerge = e[0] != '0';
     if (const char* e = std::getenv("LMOSEM_ZMED")) ctx->zmed = std::max(0, std::min(16, std::atoi(e)));
+    if (const char* e = std::getenv("LMOSEM_ZAMERGE")) ctx->zamerge = e[0] != '0';
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {
