@@ -203,7 +203,8 @@ int32_t lmosem_get_combine(const lmosem_ctx* ctx);
  * their window; LORs inside one of the overlapping slab-wide windows by passes A and B over
  * that window; the others by passes A and B over only the slabs they cross. The lists take
  * 4 B x events x (slabs + windows) of device memory, allocated on first use and kept with
- * the context (C4, 10^7 events, 3 + 22 + 13 lists: 1.5 GB); ENOMEM if that fails.
+ * the context (C4, 10^7 events, 3 + 22 + 13 lists: 1.5 GB); if that allocation fails the
+ * unlisted two-pass form runs instead (same result up to fp32 rounding).
  * The result is the same up to fp32 rounding. EINVAL if n_slabs < 0. */
 lmosem_status lmosem_set_slabs(lmosem_ctx* ctx, int32_t n_slabs);
 

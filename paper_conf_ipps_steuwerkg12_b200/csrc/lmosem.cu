@@ -686,17 +686,6 @@ lmosem_status launch_project_listed(lmosem_ctx* ctx, const float* evf, int64_t n
                                    const std::vector<std::pair<int, int>>& wins,
                                    const std::vector<std::pair<int, int>>& mwins) {
     const int Kf = (int)wins.size(), Km = (int)mwins.size();
-    const int nl = K + Kf + Km;
-    if (n > ctx->zlist_cap || nl > ctx->zlist_n) {
-        if (ctx->zlist) CK(cudaFree(ctx->zlist));
-        ctx->zlist = nullptr;
-        ctx->zlist_cap = 0;
-        ctx->zlist_n = 0;
-        CKA(cudaMalloc(&ctx->zlist, sizeof(int) * (size_t)n * nl));
-        ctx->zlist_cap = n;
-        ctx->zlist_n = nl;
-    }
-    if (!ctx->zcount) CKA(cudaMalloc(&ctx->zcount, sizeof(int) * lmk::kZMaxLists));
     lmk::ZClass zc{};
     zc.K = K;
     zc.Kf = Kf;
@@ -868,7 +857,29 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
             }
             if (K + (int)wins.size() + (int)mwins.size() > lmk::kZMaxLists) mwins.clear();
         }
-        if (K + (int)wins.size() <= lmk::kZMaxLists) return launch_project_listed(ctx, evf, n, K, wins, mwins);
+        // the lists (allocated on first use, kept with the context); without the memory the
+        // unlisted two-pass form runs instead
+        const int nl = K + (int)wins.size() + (int)mwins.size();
+        bool have = nl <= lmk::kZMaxLists && n <= ctx->zlist_cap && nl <= ctx->zlist_n && ctx->zcount;
+        if (!have && nl <= lmk::kZMaxLists) {
+            if (ctx->zlist) CK(cudaFree(ctx->zlist));
+            ctx->zlist = nullptr;
+            ctx->zlist_cap = 0;
+            ctx->zlist_n = 0;
+            if (cudaMalloc(&ctx->zlist, sizeof(int) * (size_t)n * nl) == cudaSuccess) {
+                ctx->zlist_cap = n;
+                ctx->zlist_n = nl;
+            } else {
+                (void)cudaGetLastError();  // out of memory is not sticky
+                ctx->zlist = nullptr;
+            }
+            if (!ctx->zcount && cudaMalloc(&ctx->zcount, sizeof(int) * lmk::kZMaxLists) != cudaSuccess) {
+                (void)cudaGetLastError();
+                ctx->zcount = nullptr;
+            }
+            have = ctx->zlist && ctx->zcount;
+        }
+        if (have) return launch_project_listed(ctx, evf, n, K, wins, mwins);
     }
     not_kernel(ctx);
     CK(cudaMemsetAsync(ctx->fp_acc, 0, sizeof(float) * n, ctx->stream));
