@@ -440,6 +440,9 @@ constexpr int PROJ_THREADS = LMK_CTA_THREADS;
 constexpr unsigned kLorRecBytes = 80;
 __host__ __device__ constexpr bool lor_in_smem(int mode) { return mode == 2 || mode == 3; }
 __host__ __device__ constexpr size_t lor_bytes_per_warp(int mode) { return 32u * (lor_in_smem(mode) ? kLorRecBytes : 24u); }
+#ifndef LMK_PASSA_TEX
+#define LMK_PASSA_TEX 0  // z-slab pass A gathers through the texture pipe (A/B; round 1: slower)
+#endif
 #ifndef LMK_LATE_WAIT
 #define LMK_LATE_WAIT 1  // listed pass A / window launches wait for their predecessor at exit (A/B)
 #endif
@@ -524,7 +527,8 @@ __global__ void __launch_bounds__(proj_threads<MODE>(), proj_min_blocks<MODE>())
                                                              int gdiv, ListArg la) {
     constexpr bool kGather = MODE <= 2 || MODE >= 5;  // forward projection in this launch
     constexpr bool kScatter = MODE == 0 || MODE >= 3;  // back-projection
-    constexpr bool kTex = MODE >= 5;  // gathers of f through the texture path
+    // gathers of f through the texture path (pass A too with LMK_PASSA_TEX, A/B builds only)
+    constexpr bool kTex = MODE >= 5 || (MODE == 2 && LMK_PASSA_TEX);
     extern __shared__ __align__(16) int2 smem_path[];
     const int lane = threadIdx.x & 31;
     const int wib = threadIdx.x >> 5;
