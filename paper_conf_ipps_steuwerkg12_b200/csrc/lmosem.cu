@@ -113,6 +113,7 @@ struct lmosem_ctx {
     int zmerge = 1;            // the windows of a coarse slab in one launch (LMOSEM_ZMERGE)
     int zmed = 6;              // medium windows: stride = coarse width / zmed (LMOSEM_ZMED; 0: none)
     int zamerge = 0;           // pass A of all coarse slabs in shared launches (LMOSEM_ZAMERGE)
+    int zmwin = 0;             // medium window width in voxels (LMOSEM_ZMWIN; 0: 1.36 x the widest coarse slab)
     int* zlist = nullptr;      // lists, zlist_cap indices each
     int* zcount = nullptr;     // their lengths (kZMaxLists)
     int64_t zlist_cap = 0;
@@ -849,7 +850,11 @@ lmosem_status launch_project(lmosem_ctx* ctx, const lmosem_event* ev, int64_t n,
         // the LORs that leave every fine window but fit one coarse-slab width: passes A and B
         // over that one window instead of over each coarse slab they meet (with what is left
         // of the list budget; none if it does not fit)
-        const int Wm = 2 * ((max_slab_extent(na, K) + 1) / 2);
+        // default width 1.36 x the widest coarse slab (C4: 256 voxels, f or c of a window 95 MB;
+        // measured 188 / 210 / 256 / 262 / 270 / 290 / 340: 21.31 / 21.33 / 20.93 / 20.96 /
+        // 21.10 / 22.28 / 24.64 ms per subset, profiles/r02_zmwin_ab)
+        const int Wm = ctx->zmwin > 0 ? std::min(na, 2 * ((ctx->zmwin + 1) / 2))
+                                      : std::min(na, 2 * (int)(0.68 * max_slab_extent(na, K) + 0.5));
         if (ctx->zmed > 0 && K > 1 && Wm < na) {
             for (int S = 2 * std::max(1, Wm / (2 * ctx->zmed));; S += 2) {
                 make(mwins, Wm, S);
@@ -1448,6 +1453,7 @@ lmosem_status init_ctx(lmosem_ctx** out, const int32_t dims[3], const double vox
     if (const char* e = std::getenv("LMOSEM_ZMERGE")) ctx->zmerge = e[0] != '0';
     if (const char* e = std::getenv("LMOSEM_ZMED")) ctx->zmed = std::max(0, std::min(16, std::atoi(e)));
     if (const char* e = std::getenv("LMOSEM_ZAMERGE")) ctx->zamerge = e[0] != '0';
+    if (const char* e = std::getenv("LMOSEM_ZMWIN")) ctx->zmwin = std::max(0, std::atoi(e));
     if (const char* e = std::getenv("LMOSEM_WIDE_N")) ctx->wide_n = std::max(0LL, std::atoll(e));
     if (const char* e = std::getenv("LMOSEM_DEBUG_STALL_MS")) ctx->debug_stall_ms = std::max(0, std::min(60000, std::atoi(e)));
     if (ctx->debug_stall_ms > 0) {
